@@ -1,0 +1,165 @@
+/*
+ * mcm.h -- C ABI of the B200 (sm_100a) push-relabel maximum-cardinality
+ * bipartite matching library (Deveci, Kaya, Ucar, Catalyurek, ICPP 2013).
+ *
+ * Citations: P:a-b = lines a..b of the paper text (PAPER.md, LF numbering).
+ *
+ * Problem.  G = (V_R u V_C, E) bipartite; rows V_R = V1 (m of them),
+ * columns V_C = V2 (n of them), matrix view P:115-118.  A matching M is a set of
+ * vertex-disjoint edges; mcm_solve returns a maximum-cardinality matching
+ * (|M| >= |M'| for every matching M').
+ *
+ * Method.  G-PR (Alg. 7): cheap initial matching, then a
+ * loop of lock- and atomic-free concurrent push / double-push steps over the
+ * active-column worklist (Alg. 8/9, worklist P:532-555, shrink
+ * P:656-701), with periodic global relabelling by a level-synchronous BFS from the
+ * unmatched rows (Alg. 4/5) scheduled by GETITERGR, gap
+ * relabelling, and a final FIXMATCHING pass.  The whole loop
+ * runs on the device in one persistent kernel; the only host synchronisation of a
+ * solve is the final read of the cardinality.
+ *
+ * Conventions.  All ids are int32, 0-based.  Graph input is the CSR of the m x n
+ * pattern (row u -> columns).  Unsorted adjacency and duplicate entries are
+ * accepted (they change tie-breaks only).  m = 0, n = 0 or nnz = 0 is valid.
+ * Limits: m + n + 2 < 2^31 and nnz < 2^31, else MCM_EINVAL.
+ *
+ * Memory.  The library performs NO device allocation: the caller provides one
+ * device workspace of at least mcm_workspace_bytes() bytes (e.g. a torch uint8
+ * tensor) that must outlive the handle.  indptr/indices are borrowed only for the
+ * duration of mcm_create (they are copied and transposed into the workspace).
+ * The handle itself is a small host object.
+ *
+ * Streams.  Every call enqueues its device work on the given stream; nothing
+ * touches the legacy default stream or synchronises the device.  mcm_create and
+ * mcm_solve synchronise `stream` once each (to return an error code / the
+ * cardinality).  A handle is bound to the device current at mcm_create; calling
+ * it with another device current returns MCM_EDEVICE.  One handle per host
+ * thread (handles are not thread-safe).  After MCM_ECUDA the handle is poisoned:
+ * every later call returns MCM_ECUDA.
+ */
+#ifndef MCM_H_
+#define MCM_H_
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct mcm_ctx *mcm_handle_t;
+typedef void *mcm_stream_t; /* a cudaStream_t (NULL = legacy default stream) */
+
+enum {
+  MCM_OK = 0,
+  MCM_EINVAL = -1,    /* bad argument or malformed CSR (see mcm_create) */
+  MCM_ECUDA = -2,     /* a CUDA runtime call failed; the handle is poisoned */
+  MCM_ENOMEM = -3,    /* workspace smaller than mcm_workspace_bytes() */
+  MCM_EDEVICE = -4,   /* called with a different current device than at create */
+  MCM_ENOCONV = -5,   /* iteration cap (options.max_loops) exceeded */
+  MCM_EINTERNAL = -6  /* internal consistency check failed (a bug) */
+};
+
+/* GR frequency strategy: adaptive = next GR after k*maxLevel loops,
+ * fixed = every k loops. */
+enum { MCM_GR_ADAPTIVE = 0, MCM_GR_FIXED = 1 };
+
+/* Initial matching: cheap greedy on the device (reading R13), the
+ * caller's matching in rmatch/cmatch (must be a valid matching whose two arrays
+ * are mutually consistent), or empty. */
+enum { MCM_INIT_GREEDY = 0, MCM_INIT_GIVEN = 1, MCM_INIT_EMPTY = 2 };
+
+typedef struct {
+  double k;             /* GR frequency.  Adaptive: next GR after max(1, ceil(k*maxLevel))
+                           loops; fixed: every max(1, (int)k) loops.  Default 0.7
+                           (P:753-755). */
+  int32_t gr_strategy;  /* MCM_GR_ADAPTIVE (default) or MCM_GR_FIXED */
+  int32_t shrink_min;   /* compact the worklist after a GR when |Ac| >= shrink_min
+                           (G-PR-SHRKRNL); default 512;
+                           < 0: never (G-PR-NoShr). */
+  int32_t init;         /* MCM_INIT_GREEDY (default), MCM_INIT_GIVEN, MCM_INIT_EMPTY */
+  int32_t gap;          /* gap relabelling (reading R14): 0 off (default), 1 on */
+  int32_t final_check;  /* 1 (default): exactness guard -- one GR after termination;
+                           any unmatched column it reaches is re-activated (R16). */
+  int32_t dead_skip;    /* 1 (default): an active column whose label is already
+                           >= m+n dies without scanning Gamma(v) (R19). */
+  int32_t tail_max;     /* worklists of at most this many slots run on one CTA with
+                           CTA barriers instead of grid barriers (0 = off); default 2048 */
+  int32_t compact_every;/* 1: compact the worklist at every fix step (an option beyond
+                           the paper's post-GR shrink); default 0 */
+  int32_t grid_ctas;    /* CTAs of the persistent kernel; 0 (default) = all co-resident */
+  int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
+} mcm_options_t;
+
+typedef struct {
+  int64_t loops;             /* iterations of Alg. 7's while loop */
+  int64_t gr_count;          /* global relabels (incl. the guard GR) */
+  int64_t gr_levels;         /* sum over GRs of BFS row levels */
+  int64_t pushes;            /* successful single/double pushes */
+  int64_t blocked;           /* pushes refused by the iA test (Alg. 9 l.13) */
+  int64_t dead;              /* columns declared unmatchable (mu = -2) */
+  int64_t edges_scanned;     /* neighbours read by the push scans */
+  int64_t slots;             /* worklist slots visited by fix steps */
+  int64_t shrinks;           /* SHRKRNL compactions */
+  int64_t gaps;              /* gap relabels applied */
+  int64_t guard_reactivated; /* columns re-activated by the exactness guard */
+  int64_t fixed_cols;        /* columns reset by FIXMATCHING */
+  int64_t init_card;         /* |M0| */
+  int64_t card;              /* |M| returned */
+  int64_t tail_loops;        /* loops run in the single-CTA tail mode */
+  int64_t grid_barriers;     /* grid-wide barriers executed */
+  double ms_init;            /* device time: initial matching + worklist build */
+  double ms_gr;              /* device time in global relabels */
+  double ms_loop;            /* device time in fix + push steps */
+  double ms_total;           /* device time of the whole solve kernel */
+  double ms_setup;           /* mcm_create: validation + copy + transpose (host-timed) */
+  int32_t grid_ctas, threads_per_cta;
+} mcm_stats_t;
+
+/* Fill *o with the defaults above. */
+void mcm_default_options(mcm_options_t *o);
+
+/* Bytes of device workspace a handle for an (m, n, nnz) graph needs (256-B aligned
+ * sub-buffers).  Returns 0 when the sizes are out of range. */
+size_t mcm_workspace_bytes(int32_t m, int32_t n, int64_t nnz, const mcm_options_t *o);
+
+/* Validate the CSR (indptr[0] = 0, non-decreasing, indptr[m] = nnz, 0 <= indices
+ * < n; one O(m + nnz) device pass), copy it and build the CSC transpose in the
+ * workspace.  indptr (m+1) and indices (nnz) are DEVICE pointers.  o = NULL means
+ * defaults.  Returns MCM_OK and *out, or an error code (no handle is created). */
+int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz, void *workspace,
+               size_t ws_bytes, mcm_stream_t stream, const mcm_options_t *o, mcm_handle_t *out);
+
+/* Run G-PR.  rmatch (m) and cmatch (n) are caller-owned DEVICE int32 buffers,
+ * written on return: rmatch[u] = column or -1, cmatch[v] = row or -1, mutually
+ * consistent (FIXMATCHING: the internal -2 "dead" mark never escapes).
+ * With MCM_INIT_GIVEN they are also read as the initial matching.  Returns the
+ * cardinality (>= 0) or a negative error code.  Synchronises `stream` once. */
+int64_t mcm_solve(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t *cmatch);
+
+/* Global relabel (Alg. 4/5) of a given matching: rmatch (m) and cmatch
+ * (n) are DEVICE inputs with the paper's mu conventions (column entries may be
+ * stale or -2; rows are authoritative); writes psi_row (m) and psi_col
+ * (n) (DEVICE) = exact alternating BFS distance from the unmatched rows, m+n when
+ * unreached.  Returns maxLevel = (deepest row level) + 2 (Alg. 4's final cLevel),
+ * or a negative error code.  *reached_free (may be NULL) = number of columns that
+ * are not matched but got a finite label (> 0 iff an augmenting path exists). */
+int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,
+                           int32_t *psi_row, int32_t *psi_col, int64_t *reached_free);
+
+/* Replace the options of a handle (takes effect at the next solve). */
+int mcm_set_options(mcm_handle_t h, const mcm_options_t *o);
+int mcm_set_k(mcm_handle_t h, double k);
+
+/* Statistics of the last mcm_solve. */
+int mcm_get_stats(mcm_handle_t h, mcm_stats_t *out);
+
+/* Free the host handle (the workspace stays the caller's). */
+int mcm_destroy(mcm_handle_t h);
+
+const char *mcm_strerror(int code);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* MCM_H_ */

@@ -1,0 +1,233 @@
+"""B200-native push-relabel maximum-cardinality bipartite matching (G-PR,
+Deveci, Kaya, Ucar, Catalyurek, ICPP 2013) -- thin Python binding of the C ABI in
+``include/mcm.h``.
+
+This module only marshals arguments: every step of the method runs in the CUDA
+library ``libmcm.so`` (built in-tree by ``__graft_entry__.build()``).  PyTorch
+supplies device memory and streams.  There is no CPU fallback: importing works
+anywhere, but every call raises if the library or a CUDA device is missing.
+
+Names follow include/mcm.h:
+
+* :func:`mcm_default_options`, :func:`mcm_workspace_bytes`
+* :class:`Matcher` -- ``mcm_create`` / ``mcm_solve`` / ``mcm_global_relabel`` /
+  ``mcm_set_options`` / ``mcm_get_stats`` / ``mcm_destroy`` on one graph
+* :func:`solve` -- create + solve in one call: ``(card, rmatch, cmatch)``
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+__all__ = ["Options", "Stats", "Matcher", "solve", "lib", "mcm_default_options", "mcm_workspace_bytes",
+           "MCMError", "LIB_PATH"]
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libmcm.so")
+
+MCM_OK, MCM_EINVAL, MCM_ECUDA, MCM_ENOMEM, MCM_EDEVICE, MCM_ENOCONV, MCM_EINTERNAL = 0, -1, -2, -3, -4, -5, -6
+MCM_GR_ADAPTIVE, MCM_GR_FIXED = 0, 1
+MCM_INIT_GREEDY, MCM_INIT_GIVEN, MCM_INIT_EMPTY = 0, 1, 2
+
+
+class Options(ctypes.Structure):
+    """mcm_options_t"""
+
+    _fields_ = [
+        ("k", ctypes.c_double),
+        ("gr_strategy", ctypes.c_int32),
+        ("shrink_min", ctypes.c_int32),
+        ("init", ctypes.c_int32),
+        ("gap", ctypes.c_int32),
+        ("final_check", ctypes.c_int32),
+        ("dead_skip", ctypes.c_int32),
+        ("tail_max", ctypes.c_int32),
+        ("compact_every", ctypes.c_int32),
+        ("grid_ctas", ctypes.c_int32),
+        ("max_loops", ctypes.c_int64),
+    ]
+
+
+class Stats(ctypes.Structure):
+    """mcm_stats_t"""
+
+    _fields_ = [(f, ctypes.c_int64) for f in (
+        "loops", "gr_count", "gr_levels", "pushes", "blocked", "dead", "edges_scanned", "slots", "shrinks", "gaps",
+        "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers")] + [
+        (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
+        ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
+
+    def as_dict(self):
+        return {f: getattr(self, f) for f, _ in self._fields_}
+
+
+class MCMError(RuntimeError):
+    def __init__(self, code, what=""):
+        self.code = code
+        super().__init__(f"{what}: {lib().mcm_strerror(code).decode()} (code {code})")
+
+
+_lib = None
+
+
+def lib():
+    """Load libmcm.so (fails loudly when it has not been built)."""
+    global _lib
+    if _lib is None:
+        if not os.path.exists(LIB_PATH):
+            raise ImportError(f"{LIB_PATH} missing: run `python -c 'import __graft_entry__ as g; g.build()'`")
+        L = ctypes.CDLL(LIB_PATH)
+        vp, i32, i64, sz = ctypes.c_void_p, ctypes.c_int32, ctypes.c_int64, ctypes.c_size_t
+        P = ctypes.POINTER
+        L.mcm_default_options.argtypes = [P(Options)]
+        L.mcm_default_options.restype = None
+        L.mcm_workspace_bytes.argtypes = [i32, i32, i64, P(Options)]
+        L.mcm_workspace_bytes.restype = sz
+        L.mcm_create.argtypes = [vp, vp, i32, i32, i64, vp, sz, vp, P(Options), P(vp)]
+        L.mcm_create.restype = ctypes.c_int
+        L.mcm_solve.argtypes = [vp, vp, vp, vp]
+        L.mcm_solve.restype = i64
+        L.mcm_global_relabel.argtypes = [vp, vp, vp, vp, vp, vp, P(i64)]
+        L.mcm_global_relabel.restype = i64
+        L.mcm_set_options.argtypes = [vp, P(Options)]
+        L.mcm_set_options.restype = ctypes.c_int
+        L.mcm_set_k.argtypes = [vp, ctypes.c_double]
+        L.mcm_set_k.restype = ctypes.c_int
+        L.mcm_get_stats.argtypes = [vp, P(Stats)]
+        L.mcm_get_stats.restype = ctypes.c_int
+        L.mcm_destroy.argtypes = [vp]
+        L.mcm_destroy.restype = ctypes.c_int
+        L.mcm_strerror.argtypes = [ctypes.c_int]
+        L.mcm_strerror.restype = ctypes.c_char_p
+        _lib = L
+    return _lib
+
+
+def mcm_default_options(**overrides) -> Options:
+    o = Options()
+    lib().mcm_default_options(ctypes.byref(o))
+    for k, v in overrides.items():
+        if k == "gr_strategy" and isinstance(v, str):
+            v = {"adaptive": MCM_GR_ADAPTIVE, "fixed": MCM_GR_FIXED}[v]
+        if k == "init" and isinstance(v, str):
+            v = {"greedy": MCM_INIT_GREEDY, "given": MCM_INIT_GIVEN, "empty": MCM_INIT_EMPTY}[v]
+        if not hasattr(o, k):
+            raise TypeError(f"unknown option {k}")
+        setattr(o, k, v)
+    return o
+
+
+def mcm_workspace_bytes(m: int, n: int, nnz: int, opts: Options | None = None) -> int:
+    return lib().mcm_workspace_bytes(m, n, nnz, ctypes.byref(opts) if opts is not None else None)
+
+
+def _torch():
+    import torch
+
+    return torch
+
+
+def _stream_ptr(stream):
+    torch = _torch()
+    s = stream if stream is not None else torch.cuda.current_stream()
+    return ctypes.c_void_p(s.cuda_stream)
+
+
+def _dev_i32(t, name, length):
+    torch = _torch()
+    if not isinstance(t, torch.Tensor) or not t.is_cuda:
+        raise TypeError(f"{name} must be a CUDA tensor (no CPU fallback)")
+    if t.dtype != torch.int32 or not t.is_contiguous() or t.numel() != length:
+        raise ValueError(f"{name}: need a contiguous int32 tensor of {length} elements")
+    return ctypes.c_void_p(t.data_ptr() if length else 0)
+
+
+class Matcher:
+    """One graph on one device: mcm_create at construction, mcm_destroy on close().
+
+    indptr (m+1) / indices (nnz): int32 CUDA tensors of the CSR (rows -> columns).
+    The workspace is a torch uint8 tensor owned by this object."""
+
+    def __init__(self, indptr, indices, m: int, n: int, stream=None, **opts):
+        torch = _torch()
+        for name, t in (("indptr", indptr), ("indices", indices)):
+            if not isinstance(t, torch.Tensor) or not t.is_cuda:
+                raise TypeError(f"{name} must be a CUDA tensor (no CPU fallback)")
+        self.m, self.n = int(m), int(n)
+        self.nnz = int(indices.numel())
+        self.opts = mcm_default_options(**opts)
+        self.device = indptr.device
+        need = mcm_workspace_bytes(self.m, self.n, self.nnz, self.opts)
+        if need == 0:
+            raise MCMError(MCM_EINVAL, "mcm_workspace_bytes")
+        with torch.cuda.device(self.device):
+            self.workspace = torch.empty(need, dtype=torch.uint8, device=self.device)
+            h = ctypes.c_void_p()
+            rc = lib().mcm_create(_dev_i32(indptr, "indptr", self.m + 1), _dev_i32(indices, "indices", self.nnz),
+                                  self.m, self.n, self.nnz, ctypes.c_void_p(self.workspace.data_ptr()), need,
+                                  _stream_ptr(stream), ctypes.byref(self.opts), ctypes.byref(h))
+        if rc != MCM_OK:
+            raise MCMError(rc, "mcm_create")
+        self._h = h
+
+    def set_options(self, **opts):
+        o = mcm_default_options(**{**{f: getattr(self.opts, f) for f, _ in Options._fields_}, **opts})
+        rc = lib().mcm_set_options(self._h, ctypes.byref(o))
+        if rc != MCM_OK:
+            raise MCMError(rc, "mcm_set_options")
+        self.opts = o
+
+    def solve(self, rmatch=None, cmatch=None, stream=None):
+        """mcm_solve -> (card, rmatch, cmatch) (int32 CUDA tensors)."""
+        torch = _torch()
+        if rmatch is None:
+            rmatch = torch.empty(self.m, dtype=torch.int32, device=self.device)
+        if cmatch is None:
+            cmatch = torch.empty(self.n, dtype=torch.int32, device=self.device)
+        with torch.cuda.device(self.device):
+            card = lib().mcm_solve(self._h, _stream_ptr(stream), _dev_i32(rmatch, "rmatch", self.m),
+                                   _dev_i32(cmatch, "cmatch", self.n))
+        if card < 0:
+            raise MCMError(int(card), "mcm_solve")
+        return int(card), rmatch, cmatch
+
+    def global_relabel(self, rmatch, cmatch, stream=None):
+        """mcm_global_relabel -> (max_level, psi_row, psi_col, reached_free)."""
+        torch = _torch()
+        pr = torch.empty(self.m, dtype=torch.int32, device=self.device)
+        pc = torch.empty(self.n, dtype=torch.int32, device=self.device)
+        rf = ctypes.c_int64(0)
+        with torch.cuda.device(self.device):
+            ml = lib().mcm_global_relabel(self._h, _stream_ptr(stream), _dev_i32(rmatch, "rmatch", self.m),
+                                          _dev_i32(cmatch, "cmatch", self.n), _dev_i32(pr, "psi_row", self.m),
+                                          _dev_i32(pc, "psi_col", self.n), ctypes.byref(rf))
+        if ml < 0:
+            raise MCMError(int(ml), "mcm_global_relabel")
+        return int(ml), pr, pc, int(rf.value)
+
+    def stats(self) -> dict:
+        s = Stats()
+        rc = lib().mcm_get_stats(self._h, ctypes.byref(s))
+        if rc != MCM_OK:
+            raise MCMError(rc, "mcm_get_stats")
+        return s.as_dict()
+
+    def close(self):
+        if getattr(self, "_h", None):
+            lib().mcm_destroy(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def solve(indptr, indices, m: int, n: int, stream=None, **opts):
+    """Create + solve: ``(card, rmatch, cmatch)`` with rmatch/cmatch int32 CUDA tensors."""
+    mt = Matcher(indptr, indices, m, n, stream=stream, **opts)
+    try:
+        return mt.solve(stream=stream)
+    finally:
+        mt.close()

@@ -1,0 +1,387 @@
+// api.cu -- the C ABI of include/mcm.h: workspace layout, graph ingest (validate,
+// copy, CSC transpose) and the cooperative launch of the persistent G-PR kernel.
+#include <cuda_runtime.h>
+#include <chrono>
+#include <cmath>
+#include <cstdio>
+#include <cstring>
+#include <cstdlib>
+#include <new>
+#include <memory>
+#include <algorithm>
+
+#include "../../include/mcm.h"
+#include "solve.cuh"
+
+using namespace mcm;
+
+namespace {
+
+constexpr int SCAN_B = 2048;  // items per scan block
+constexpr int MAX_CTAS = 4096;
+
+size_t align256(size_t x) { return (x + 255) & ~(size_t)255; }
+
+struct Layout {
+  size_t ctrl, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, dbg, total;
+};
+
+Layout layout(int32_t m, int32_t n, int64_t nnz) {
+  Layout L;
+  size_t o = 0;
+  auto take = [&](size_t bytes) { size_t r = o; o += align256(bytes > 0 ? bytes : 1); return r; };
+  size_t mx = (size_t)(m > n ? m : n) + 1;
+  L.ctrl = take(sizeof(Ctrl));
+  L.rptr = take(sizeof(int) * ((size_t)m + 1));
+  L.radj = take(sizeof(int) * (size_t)nnz);
+  L.cptr = take(sizeof(int) * ((size_t)n + 1));
+  L.cadj = take(sizeof(int) * (size_t)nnz);
+  L.rowst = take(sizeof(u64) * (size_t)m);
+  L.colst = take(sizeof(u64) * (size_t)n);
+  L.iA = take(sizeof(int) * (size_t)n);
+  L.wl0 = take(sizeof(int) * (size_t)n);
+  L.wl1 = take(sizeof(int) * (size_t)n);
+  for (int i = 0; i < 4; i++) L.q[i] = take(sizeof(int) * mx);
+  L.ctacnt = take(sizeof(int) * MAX_CTAS);
+  L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
+  L.dbg = take(sizeof(int) * ((size_t)n + 1));
+  L.total = o;
+  return L;
+}
+
+// ---------------------------------------------------------------- setup kernels
+__global__ void k_validate(const int *indptr, const int *indices, int m, int n, long long nnz, int *err) {
+  long long g = (long long)blockIdx.x * blockDim.x + threadIdx.x, G = (long long)gridDim.x * blockDim.x;
+  if (g == 0) {
+    if (indptr[0] != 0 || (long long)indptr[m] != nnz) atomicOr(err, 1);
+  }
+  for (long long u = g; u < m; u += G)
+    if (indptr[u] > indptr[u + 1]) atomicOr(err, 2);
+  for (long long e = g; e < nnz; e += G) {
+    int v = indices[e];
+    if (v < 0 || v >= n) atomicOr(err, 4);
+  }
+}
+
+// count column degrees into cnt[0..n)
+__global__ void k_count(const int *indices, long long nnz, int *cnt) {
+  long long g = (long long)blockIdx.x * blockDim.x + threadIdx.x, G = (long long)gridDim.x * blockDim.x;
+  for (long long e = g; e < nnz; e += G) atomicAdd(cnt + __ldg(indices + e), 1);
+}
+
+// exclusive scan, 3 phases: block sums, scan of block sums (one CTA), block scans
+__global__ void k_scan_sums(const int *in, int len, int *bsum) {
+  __shared__ long long red[32];
+  int b = blockIdx.x, lo = b * SCAN_B;
+  long long s = 0;
+  for (int i = lo + threadIdx.x; i < min(len, lo + SCAN_B); i += blockDim.x) s += in[i];
+  for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+  if ((threadIdx.x & 31) == 0) red[threadIdx.x >> 5] = s;
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    long long t = 0;
+    for (int w = 0; w < (int)(blockDim.x >> 5); w++) t += red[w];
+    bsum[b] = (int)t;
+  }
+}
+__global__ void k_scan_bsum(int *bsum, int nb) {
+  // one CTA of 1024 threads, sequential chunks
+  __shared__ int s[1024];
+  __shared__ int carry;
+  if (threadIdx.x == 0) carry = 0;
+  __syncthreads();
+  for (int base = 0; base < nb; base += 1024) {
+    int i = base + threadIdx.x;
+    int x = i < nb ? bsum[i] : 0;
+    s[threadIdx.x] = x;
+    __syncthreads();
+    for (int o = 1; o < 1024; o <<= 1) {
+      int y = threadIdx.x >= o ? s[threadIdx.x - o] : 0;
+      __syncthreads();
+      s[threadIdx.x] += y;
+      __syncthreads();
+    }
+    if (i < nb) bsum[i] = carry + s[threadIdx.x] - x;  // exclusive
+    __syncthreads();
+    if (threadIdx.x == 1023) carry += s[1023];
+    __syncthreads();
+  }
+}
+__global__ void k_scan_apply(const int *in, int len, const int *bsum, int *out, int total_slot) {
+  // block of 1024 threads, SCAN_B = 2 items per thread
+  __shared__ int s[1024];
+  int b = blockIdx.x, lo = b * SCAN_B;
+  int i0 = lo + 2 * threadIdx.x, i1 = i0 + 1;
+  int x0 = i0 < len ? in[i0] : 0, x1 = i1 < len ? in[i1] : 0;
+  s[threadIdx.x] = x0 + x1;
+  __syncthreads();
+  for (int o = 1; o < 1024; o <<= 1) {
+    int y = threadIdx.x >= o ? s[threadIdx.x - o] : 0;
+    __syncthreads();
+    s[threadIdx.x] += y;
+    __syncthreads();
+  }
+  int ex = bsum[b] + s[threadIdx.x] - x0 - x1;
+  if (i0 < len) out[i0] = ex;
+  if (i1 < len) out[i1] = ex + x0;
+  if (total_slot >= 0 && b == gridDim.x - 1 && threadIdx.x == 1023) out[total_slot] = ex + x0 + x1;
+}
+
+// scatter rows into Gamma(v) lists: thread per short row, warp per long row
+__global__ void k_scatter(const int *rptr, const int *radj, int m, int *cursor, int *cadj) {
+  int lane = threadIdx.x & 31;
+  long long gw = ((long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+  long long NW = ((long long)gridDim.x * blockDim.x) >> 5;
+  for (long long b = gw * 32; b < m; b += NW * 32) {
+    int u = (int)(b + lane);
+    int s = 0, e = 0;
+    if (u < m) { s = rptr[u]; e = rptr[u + 1]; }
+    if (u < m && e - s <= 32)
+      for (int j = s; j < e; j++) cadj[atomicAdd(cursor + radj[j], 1)] = u;
+    unsigned big = __ballot_sync(0xffffffffu, u < m && e - s > 32);
+    while (big) {
+      int bl = __ffs(big) - 1;
+      big &= big - 1;
+      int ub = __shfl_sync(0xffffffffu, u, bl), sb = __shfl_sync(0xffffffffu, s, bl),
+          eb = __shfl_sync(0xffffffffu, e, bl);
+      for (int j = sb + lane; j < eb; j += 32) cadj[atomicAdd(cursor + radj[j], 1)] = ub;
+    }
+  }
+}
+
+}  // namespace
+
+struct mcm_ctx {
+  int dev = 0, sms = 0;
+  int32_t m = 0, n = 0;
+  int64_t nnz = 0;
+  mcm_options_t opt;
+  char *ws = nullptr;
+  Layout L;
+  int grid = 0, max_grid = 0;
+  bool poisoned = false;
+  mcm_stats_t stats;
+  double ms_setup = 0;
+  Ctrl host_ctrl;
+};
+
+#define CK(x)                                  \
+  do {                                         \
+    cudaError_t e_ = (x);                      \
+    if (e_ != cudaSuccess) {                   \
+      if (h) h->poisoned = true;               \
+      last_cuda_error = e_;                    \
+      return MCM_ECUDA;                        \
+    }                                          \
+  } while (0)
+
+static thread_local cudaError_t last_cuda_error = cudaSuccess;
+
+extern "C" {
+
+void mcm_default_options(mcm_options_t *o) {
+  if (!o) return;
+  memset(o, 0, sizeof(*o));
+  o->k = 0.7;
+  o->gr_strategy = MCM_GR_ADAPTIVE;
+  o->shrink_min = 512;
+  o->init = MCM_INIT_GREEDY;
+  o->gap = 0;
+  o->final_check = 1;
+  o->dead_skip = 1;
+  o->tail_max = 2048;
+  o->compact_every = 0;
+  o->grid_ctas = 0;
+  o->max_loops = 0;
+}
+
+static bool sizes_ok(int32_t m, int32_t n, int64_t nnz) {
+  return m >= 0 && n >= 0 && nnz >= 0 && (int64_t)m + n + 2 < ((int64_t)1 << 31) && nnz < ((int64_t)1 << 31);
+}
+
+size_t mcm_workspace_bytes(int32_t m, int32_t n, int64_t nnz, const mcm_options_t *) {
+  if (!sizes_ok(m, n, nnz)) return 0;
+  return layout(m, n, nnz).total;
+}
+
+const char *mcm_strerror(int code) {
+  switch (code) {
+    case MCM_OK: return "ok";
+    case MCM_EINVAL: return "invalid argument or malformed CSR";
+    case MCM_ECUDA: return cudaGetErrorString(last_cuda_error);
+    case MCM_ENOMEM: return "workspace too small";
+    case MCM_EDEVICE: return "wrong current device for this handle";
+    case MCM_ENOCONV: return "iteration cap exceeded";
+    case MCM_EINTERNAL: return "internal error";
+    default: return "unknown error";
+  }
+}
+
+static int check_opts(const mcm_options_t *o) {
+  if (!o) return MCM_OK;
+  if (!(o->k > 0) || !std::isfinite(o->k)) return MCM_EINVAL;
+  if (o->gr_strategy != MCM_GR_ADAPTIVE && o->gr_strategy != MCM_GR_FIXED) return MCM_EINVAL;
+  if (o->init < 0 || o->init > 2) return MCM_EINVAL;
+  if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->max_loops < 0) return MCM_EINVAL;
+  return MCM_OK;
+}
+
+int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz, void *workspace,
+               size_t ws_bytes, mcm_stream_t stream_, const mcm_options_t *o, mcm_handle_t *out) {
+  mcm_ctx *h = nullptr;
+  if (!out || !sizes_ok(m, n, nnz) || !indptr || (nnz > 0 && !indices) || !workspace) return MCM_EINVAL;
+  if (check_opts(o) != MCM_OK) return MCM_EINVAL;
+  *out = nullptr;
+  Layout L = layout(m, n, nnz);
+  if (ws_bytes < L.total) return MCM_ENOMEM;
+  cudaStream_t st = (cudaStream_t)stream_;
+  auto t0 = std::chrono::steady_clock::now();
+  h = new (std::nothrow) mcm_ctx();
+  if (!h) return MCM_ENOMEM;
+  std::unique_ptr<mcm_ctx> guard(h);
+  h->m = m; h->n = n; h->nnz = nnz; h->L = L; h->ws = (char *)workspace;
+  if (o) h->opt = *o; else mcm_default_options(&h->opt);
+  CK(cudaGetDevice(&h->dev));
+  CK(cudaDeviceGetAttribute(&h->sms, cudaDevAttrMultiProcessorCount, h->dev));
+  int per_sm = 0;
+  CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel, NT, 0));
+  if (per_sm < 1) return MCM_EINTERNAL;
+  h->max_grid = h->sms * (per_sm > 2 ? 2 : per_sm);
+  if (h->max_grid > MAX_CTAS) h->max_grid = MAX_CTAS;
+
+  char *ws = h->ws;
+  Ctrl *ctrl = (Ctrl *)(ws + L.ctrl);
+  int *err = &ctrl->err;
+  CK(cudaMemsetAsync(ctrl, 0, sizeof(Ctrl), st));
+  int vb = (int)std::min<long long>(std::max<long long>((nnz + 255) / 256, (m + 255) / 256 + 1), 4096);
+  k_validate<<<vb, 256, 0, st>>>(indptr, indices, m, n, nnz, err);
+  CK(cudaGetLastError());
+  int herr = 0;
+  CK(cudaMemcpyAsync(&herr, err, sizeof(int), cudaMemcpyDeviceToHost, st));
+  CK(cudaStreamSynchronize(st));
+  if (herr) return MCM_EINVAL;
+
+  int *rptr = (int *)(ws + L.rptr), *radj = (int *)(ws + L.radj);
+  int *cptr = (int *)(ws + L.cptr), *cadj = (int *)(ws + L.cadj);
+  int *cnt = (int *)(ws + L.q[0]), *cursor = (int *)(ws + L.q[1]), *bsum = (int *)(ws + L.bsum);
+  CK(cudaMemcpyAsync(rptr, indptr, sizeof(int) * ((size_t)m + 1), cudaMemcpyDeviceToDevice, st));
+  if (nnz) CK(cudaMemcpyAsync(radj, indices, sizeof(int) * (size_t)nnz, cudaMemcpyDeviceToDevice, st));
+  // CSC by counting sort (Gamma(v) for the push, Alg. 9 l.6)
+  CK(cudaMemsetAsync(cnt, 0, sizeof(int) * ((size_t)n + 1), st));
+  if (nnz) {
+    int cb = (int)std::min<long long>((nnz + 255) / 256, 148 * 16);
+    k_count<<<cb, 256, 0, st>>>(radj, nnz, cnt);
+    CK(cudaGetLastError());
+  }
+  int nb = (n + SCAN_B - 1) / SCAN_B;
+  if (nb == 0) nb = 1;
+  k_scan_sums<<<nb, 512, 0, st>>>(cnt, n, bsum);
+  k_scan_bsum<<<1, 1024, 0, st>>>(bsum, nb);
+  k_scan_apply<<<nb, 1024, 0, st>>>(cnt, n, bsum, cptr, n);
+  CK(cudaGetLastError());
+  if (n == 0) CK(cudaMemsetAsync(cptr, 0, sizeof(int), st));
+  CK(cudaMemcpyAsync(cursor, cptr, sizeof(int) * ((size_t)n + 1), cudaMemcpyDeviceToDevice, st));
+  if (nnz) {
+    int sb = (int)std::min<long long>(((long long)m + 255) / 256, 148 * 16);
+    if (sb < 1) sb = 1;
+    k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, cursor, cadj);
+    CK(cudaGetLastError());
+  }
+  CK(cudaStreamSynchronize(st));
+  h->ms_setup = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
+  memset(&h->stats, 0, sizeof(h->stats));
+  *out = guard.release();
+  return MCM_OK;
+}
+
+static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin, const int32_t *cin, int32_t *out_r,
+                      int32_t *out_c) {
+  if (h->poisoned) return MCM_ECUDA;
+  int dev = -1;
+  CK(cudaGetDevice(&dev));
+  if (dev != h->dev) return MCM_EDEVICE;
+  const Layout &L = h->L;
+  char *ws = h->ws;
+  Params p;
+  memset(&p, 0, sizeof(p));
+  p.m = h->m; p.n = h->n; p.mode = mode;
+  p.rptr = (const int *)(ws + L.rptr); p.radj = (const int *)(ws + L.radj);
+  p.cptr = (const int *)(ws + L.cptr); p.cadj = (const int *)(ws + L.cadj);
+  p.rowst = (u64 *)(ws + L.rowst); p.colst = (u64 *)(ws + L.colst);
+  p.iA = (int *)(ws + L.iA); p.wl0 = (int *)(ws + L.wl0); p.wl1 = (int *)(ws + L.wl1);
+  p.qa = (int *)(ws + L.q[0]); p.qb = (int *)(ws + L.q[1]); p.qc = (int *)(ws + L.q[2]); p.qd = (int *)(ws + L.q[3]);
+  p.ctacnt = (int *)(ws + L.ctacnt);
+  p.ctrl = (Ctrl *)(ws + L.ctrl);
+  p.dbgbuf = (int *)(ws + L.dbg);
+  p.debug = getenv("MCM_DEBUG") ? atoi(getenv("MCM_DEBUG")) : 0;
+  const mcm_options_t &o = h->opt;
+  p.k = o.k; p.gr_fixed = o.gr_strategy == MCM_GR_FIXED; p.shrink_min = o.shrink_min; p.init = o.init;
+  p.gap = o.gap; p.final_check = o.final_check; p.dead_skip = o.dead_skip; p.tail_max = o.tail_max;
+  p.compact_every = o.compact_every;
+  p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
+  p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
+  int grid = o.grid_ctas > 0 ? std::min(o.grid_ctas, h->max_grid) : h->max_grid;
+  h->grid = grid;
+  CK(cudaMemsetAsync(p.ctrl, 0, sizeof(Ctrl), st));
+  void *args[] = {&p};
+  CK(cudaLaunchCooperativeKernel((void *)gpr_kernel, grid, NT, args, 0, st));
+  CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));
+  CK(cudaStreamSynchronize(st));
+  const Ctrl &c = h->host_ctrl;
+  mcm_stats_t &s = h->stats;
+  memset(&s, 0, sizeof(s));
+  const long long *x = c.stat;
+  s.loops = x[ST_LOOPS]; s.gr_count = x[ST_GRS]; s.gr_levels = x[ST_LEVELS]; s.pushes = x[ST_PUSHES];
+  s.blocked = x[ST_BLOCKED]; s.dead = x[ST_DEAD]; s.edges_scanned = x[ST_SCANNED]; s.slots = x[ST_SLOTS];
+  s.shrinks = x[ST_SHRINKS]; s.gaps = x[ST_GAPS]; s.guard_reactivated = x[ST_GUARD]; s.fixed_cols = x[ST_FIXED];
+  s.init_card = x[ST_INITCARD]; s.card = x[ST_CARD]; s.tail_loops = x[ST_TAILLOOPS]; s.grid_barriers = x[ST_BARRIERS];
+  s.ms_init = x[ST_NS_INIT] * 1e-6; s.ms_gr = x[ST_NS_GR] * 1e-6; s.ms_loop = x[ST_NS_LOOP] * 1e-6;
+  s.ms_total = x[ST_NS_TOTAL] * 1e-6; s.ms_setup = h->ms_setup; s.grid_ctas = grid; s.threads_per_cta = NT;
+  if (p.debug && c.dbg[0])
+    fprintf(stderr, "[mcm debug] %lld violations; first: where=%lld loop=%lld x=%lld val=%lld\n", c.dbg[0], c.dbg[1],
+            c.dbg[2], c.dbg[3], c.dbg[4]);
+  if (c.err) return c.err;
+  if (mode == MODE_RELABEL) return x[ST_MAXLEVEL];
+  return x[ST_CARD];
+}
+
+int64_t mcm_solve(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t *cmatch) {
+  if (!h) return MCM_EINVAL;
+  if ((h->m > 0 && !rmatch) || (h->n > 0 && !cmatch)) return MCM_EINVAL;
+  return launch(h, (cudaStream_t)stream, MODE_SOLVE, rmatch, cmatch, rmatch, cmatch);
+}
+
+int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,
+                           int32_t *psi_row, int32_t *psi_col, int64_t *reached_free) {
+  if (!h) return MCM_EINVAL;
+  if ((h->m > 0 && (!rmatch || !psi_row)) || (h->n > 0 && (!cmatch || !psi_col))) return MCM_EINVAL;
+  int64_t r = launch(h, (cudaStream_t)stream, MODE_RELABEL, rmatch, cmatch, psi_row, psi_col);
+  if (r >= 0 && reached_free) *reached_free = h->host_ctrl.stat[ST_REACHED_FREE];
+  return r;
+}
+
+int mcm_set_options(mcm_handle_t h, const mcm_options_t *o) {
+  if (!h || !o || check_opts(o) != MCM_OK) return MCM_EINVAL;
+  h->opt = *o;
+  return MCM_OK;
+}
+
+int mcm_set_k(mcm_handle_t h, double k) {
+  if (!h || !(k > 0) || !std::isfinite(k)) return MCM_EINVAL;
+  h->opt.k = k;
+  return MCM_OK;
+}
+
+int mcm_get_stats(mcm_handle_t h, mcm_stats_t *out) {
+  if (!h || !out) return MCM_EINVAL;
+  *out = h->stats;
+  return MCM_OK;
+}
+
+int mcm_destroy(mcm_handle_t h) {
+  if (!h) return MCM_EINVAL;
+  delete h;
+  return MCM_OK;
+}
+
+}  // extern "C"

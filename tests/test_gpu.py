@@ -1,0 +1,212 @@
+"""GPU parity tests (-m gpu): the CUDA path through the C ABI against the CPU oracle.
+
+* GR labels (deterministic): bit-exact psi_row, psi_col, maxLevel and the
+  reached-unmatched count against oracle.global_relabel (Alg. 2 / Alg. 4-5).
+* Full solves: the cardinality is unique -> bit-exact against the oracle
+  (Hopcroft-Karp == PR-FIFO) or the closed form; the matching itself is not
+  unique -> checked valid (pairs are edges, mates mutual, injective) and
+  certified maximum by a Konig cover of equal size computed on the host.
+"""
+import numpy as np
+import pytest
+
+import oracle
+import synth
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+import paper_conf_icpp_devecikuc13_b200 as pkg  # noqa: E402
+
+DEV = "cuda:0"
+
+
+def dev(g):
+    return torch.from_numpy(np.ascontiguousarray(g.indptr)).to(DEV), torch.from_numpy(
+        np.ascontiguousarray(g.indices)).to(DEV)
+
+
+def check_solve(g, mm=None, **opts):
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, **opts)
+    card, rm, cm = mt.solve()
+    st = mt.stats()
+    mt.close()
+    rm, cm = rm.cpu().numpy(), cm.cpu().numpy()
+    if mm is None:
+        mm = g.mm if g.mm is not None else oracle.hopcroft_karp(g)[0]
+    assert card == mm, (g.name, opts, card, mm, st)
+    assert oracle.check_matching(g, rm, cm) == card, (g.name, opts)
+    size, _, _ = oracle.konig_cover(g, rm, cm)
+    assert size == card, (g.name, opts, size)
+    assert st["card"] == card and st["guard_reactivated"] >= 0
+    return card, st
+
+
+# ---------------------------------------------------------------- GR, bit-exact
+def _noisy_matching(g, rng):
+    c, rm, cm = oracle.hopcroft_karp(g, init="empty")
+    rm, cm = rm.copy(), cm.copy()
+    for u in np.nonzero(rm >= 0)[0]:
+        if rng.random() < 0.3:
+            v = rm[u]
+            rm[u] = -1
+            cm[v] = u if rng.random() < 0.5 else -1  # stale column pointer or unmatched
+    dead = (cm == -1) & (rng.random(g.n) < 0.2)
+    cm[dead] = -2
+    return rm.astype(np.int32), cm.astype(np.int32)
+
+
+GR_GRAPHS = [
+    lambda: synth.config("C1", 0.2), lambda: synth.config("C2", 0.01), lambda: synth.config("C3", 0.002),
+    lambda: synth.config("C4", 1 / 512), lambda: synth.config("C5", 1 / 256), lambda: synth.complete(40, 25),
+    lambda: synth.path(2001), lambda: synth.hall_violator(2000, 100, 31, 3),
+]
+
+
+@pytest.mark.parametrize("gi", range(len(GR_GRAPHS)))
+def test_global_relabel_bit_exact(gi):
+    g = GR_GRAPHS[gi]()
+    rng = np.random.default_rng(gi)
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n)
+    for trial in range(3):
+        if trial == 0:
+            _, rm, cm = oracle.cheap_match(g)
+        elif trial == 1:
+            rm, cm = _noisy_matching(g, rng)
+        else:
+            rm, cm = np.full(g.m, -1, np.int32), np.full(g.n, -1, np.int32)
+        ml, pr, pc, rf = mt.global_relabel(torch.from_numpy(rm).to(DEV), torch.from_numpy(cm).to(DEV))
+        epr, epc, eml, erf = oracle.global_relabel(g, rm, cm)
+        assert np.array_equal(pr.cpu().numpy(), epr), (g.name, trial)
+        assert np.array_equal(pc.cpu().numpy(), epc), (g.name, trial)
+        assert ml == eml and rf == erf, (g.name, trial, ml, eml, rf, erf)
+    mt.close()
+
+
+# ---------------------------------------------------------------- solves
+SOLVE_GRAPHS = [
+    ("C1", lambda: synth.config("C1")), ("C2s", lambda: synth.config("C2", 0.01)),
+    ("C3s", lambda: synth.config("C3", 0.002)), ("C4s", lambda: synth.config("C4", 1 / 256)),
+    ("C5s", lambda: synth.config("C5", 1 / 64)), ("hall", lambda: synth.hall_violator(5000, 300, 77, 1)),
+    ("K64x40", lambda: synth.complete(64, 40)), ("P1001", lambda: synth.path(1001)),
+    ("C2000", lambda: synth.cycle(1000)), ("grid9", lambda: synth.grid_double_cover(9)),
+    ("union", lambda: synth.disjoint_union([synth.complete(7, 5), synth.path(99), synth.star(12),
+                                            synth.hall_violator(900, 40, 13, 2), synth.cycle(77)], seed=3)),
+]
+
+
+@pytest.mark.parametrize("name,mk", SOLVE_GRAPHS, ids=[s[0] for s in SOLVE_GRAPHS])
+def test_solve_default(name, mk):
+    check_solve(mk())
+
+
+OPTION_SETS = [
+    dict(k=0.3), dict(k=2.0), dict(gr_strategy="fixed", k=10), dict(gr_strategy="fixed", k=50), dict(shrink_min=-1),
+    dict(shrink_min=1), dict(compact_every=1), dict(init="empty"), dict(final_check=0), dict(dead_skip=0),
+    dict(tail_max=0), dict(tail_max=100000), dict(grid_ctas=1), dict(grid_ctas=7), dict(gap=1),
+]
+
+
+@pytest.mark.parametrize("opts", OPTION_SETS, ids=lambda o: ",".join(f"{k}={v}" for k, v in o.items()))
+def test_solve_options(opts):
+    for g in (synth.config("C1", 0.5), synth.config("C2", 0.005), synth.config("C3", 0.001),
+              synth.config("C4", 1 / 1024), synth.hall_violator(3000, 150, 41, 9)):
+        check_solve(g, **opts)
+
+
+def test_given_initial_matching():
+    g = synth.config("C2", 0.01)
+    _, rm0, cm0 = oracle.cheap_match(g)
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, init="given")
+    rm = torch.from_numpy(rm0.astype(np.int32)).to(DEV)
+    cm = torch.from_numpy(cm0.astype(np.int32)).to(DEV)
+    card, rm, cm = mt.solve(rm, cm)
+    assert mt.stats()["init_card"] == int((rm0 >= 0).sum())
+    assert card == g.n
+    assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == card
+
+
+def test_edge_cases():
+    check_solve(synth.from_pairs(0, 0, [], []), 0)
+    check_solve(synth.from_pairs(5, 0, [], []), 0)
+    check_solve(synth.from_pairs(0, 5, [], []), 0)
+    check_solve(synth.from_pairs(4, 6, [], []), 0)
+    check_solve(synth.from_pairs(1, 1, [0], [0]), 1)
+    check_solve(synth.star(1000), 1)
+    check_solve(synth.complete(1, 3000), 1)
+    check_solve(synth.from_pairs(3000, 50, np.arange(3000), np.arange(3000) % 50), 50)  # m >> n
+    check_solve(synth.from_pairs(50, 3000, np.arange(3000) % 50, np.arange(3000)), 50)  # n >> m
+
+
+def test_unsorted_duplicate_adjacency():
+    """The ABI accepts unsorted lists with duplicates (tie-breaks only)."""
+    g = synth.config("C1", 0.3)
+    rng = np.random.default_rng(5)
+    idx = g.indices.copy()
+    for u in range(g.m):
+        s, e = g.indptr[u], g.indptr[u + 1]
+        rng.shuffle(idx[s:e])
+    # duplicate every 7th entry of each row (append a copy)
+    rows, cols = [], []
+    for u in range(g.m):
+        lst = idx[g.indptr[u]: g.indptr[u + 1]].tolist()
+        lst = lst + lst[::7]
+        rows += [u] * len(lst)
+        cols += lst
+    indptr = np.zeros(g.m + 1, np.int32)
+    np.add.at(indptr, np.array(rows) + 1, 1)
+    indptr = np.cumsum(indptr).astype(np.int32)
+    gd = synth.Graph(g.m, g.n, indptr, np.array(cols, np.int32), "dup")
+    mm = oracle.hopcroft_karp(g)[0]
+    ip, ix = dev(gd)
+    card, rm, cm = pkg.solve(ip, ix, g.m, g.n)
+    assert card == mm
+    assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == mm
+
+
+def test_rejects_malformed_csr():
+    ip = torch.tensor([0, 2, 1], dtype=torch.int32, device=DEV)  # decreasing
+    ix = torch.tensor([0, 1], dtype=torch.int32, device=DEV)
+    with pytest.raises(pkg.MCMError):
+        pkg.Matcher(ip, ix, 2, 2)
+    ip = torch.tensor([0, 1, 2], dtype=torch.int32, device=DEV)
+    ix = torch.tensor([0, 7], dtype=torch.int32, device=DEV)  # column out of range
+    with pytest.raises(pkg.MCMError):
+        pkg.Matcher(ip, ix, 2, 2)
+    ip = torch.tensor([1, 1, 2], dtype=torch.int32, device=DEV)  # indptr[0] != 0
+    with pytest.raises(pkg.MCMError):
+        pkg.Matcher(ip, torch.tensor([0, 1], dtype=torch.int32, device=DEV), 2, 2)
+
+
+def test_race_stress():
+    """Every column races for the same rows (K_{a,b}, empty M0), repeated."""
+    for g in (synth.complete(128, 128), synth.complete(300, 40), synth.complete(40, 300), synth.grid_double_cover(30)):
+        for rep in range(10):
+            check_solve(g, init="empty")
+    for seed in range(30):
+        g = synth.random_small(200, 200, 0.02, seed)
+        check_solve(g, init="empty", k=0.3)
+
+
+def test_matcher_reuse_is_deterministic_in_card():
+    g = synth.config("C3", 0.004)
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n)
+    cards = {mt.solve()[0] for _ in range(5)}
+    assert cards == {g.n}
+    mt.close()
+
+
+# ---------------------------------------------------------------- full-size configs
+@pytest.mark.parametrize("name", ["C1", "C2", "C3", "C4", "C5"])
+def test_full_size_config(name):
+    """BASELINE.json sizes in the bench launch configuration (defaults, all CTAs):
+    closed-form MM (C2, C3) or the oracle's (C1, C4, C5); validity; Konig."""
+    g = synth.config(name)
+    mm = g.mm
+    if mm is None:
+        mm = oracle.hopcroft_karp(g)[0]
+    check_solve(g, mm)
