@@ -1,0 +1,416 @@
+"""bench.py -- G-PR maximum-cardinality matching throughput on B200.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config C2] [--impl ours|reference]
+
+One STEP = one pass of the whole hot path over one synthetic graph already
+resident in HBM: mcm_create (validate + copy + CSC transpose)
+followed by mcm_solve (greedy init, GRs, fix/push loop, guard, FIXMATCHING).
+Default workload: configs[1] of BASELINE.json (C2, permuted banded 1.5M x 1.5M,
+~5.47M nnz).  value = edges/s = (sum over ranks of nnz) / (max over ranks of the
+mean step time).  N > 1 (torchrun): every rank solves its own instance (seed + rank),
+no data-path collective -> "scaling": "weak".
+
+L2 (126 MB) is flushed between timed steps by writing a 512 MiB buffer outside
+the per-step CUDA events.  `e2e` repeats the measurement through the public API
+with the CSR in pinned HOST memory: H2D copy + create + solve + D2H of the
+matching inside the timed region.  `--impl reference` times the CPU oracle
+(sequential PR-FIFO with GR every 0.5(m+n) pushes, from the cheap
+matching) on the host cores: the paper's own CPU comparison algorithm.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+CONFIG_DESC = {
+    "C1": "uniform random bipartite 10,000 x 10,000, 80,000 samples (avg deg 8), seed 1",
+    "C2": "permuted banded circuit-like 1.5M x 1.5M, diag + Poisson(2.47) in +-64 + 150 rails x 2000, seed 2",
+    "C3": "road-like planted lattice 4900^2 = 24.01M x 24.01M, avg deg 2.5, seed 3",
+    "C4": "R-MAT 2^23 x 2^23, 2^27 samples (0.57,0.19,0.19,0.05), permuted, seed 4",
+    "C5": "uniform 2^21 x 2^21, 16 * 2^21 samples (avg deg 16), seed 1000+i",
+}
+METRIC = "MCM solve throughput (edges/s = nnz / (create + solve time)) per graph"
+
+
+def _peaks():
+    try:
+        return json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))
+    except Exception:
+        return None
+
+
+def _graph(name, rank):
+    import synth
+
+    if name == "C5":
+        return synth.config("C5", 1.0, index=rank)
+    g = synth.config(name)
+    if rank == 0:
+        return g
+    # an independent instance of the same recipe for rank > 0 (same distribution)
+    if name == "C1":
+        return synth.uniform(g.m, g.n, 8 * g.m, 1 + 7919 * rank, name="C1")
+    if name == "C2":
+        return synth.banded(g.n, 2.47, 64, 150, 2000, 2 + 7919 * rank, True, name="C2")
+    if name == "C3":
+        return synth.road(4900, 0.5, 0.4, 0.1, 3 + 7919 * rank, True, False, 256, name="C3")
+    if name == "C4":
+        return synth.rmat(23, 16 << 23, seed=4 + 7919 * rank, name="C4")
+    raise KeyError(name)
+
+
+class Clocks:
+    """nvidia-smi sampling during the timed region (B200_PROFILING.md clocks line)."""
+
+    FIELDS = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index):
+        self.index = index
+        self.proc = None
+        self.lines = []
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "50"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if not self.proc:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        time.sleep(0.06)
+        self.proc.terminate()
+        try:
+            self.proc.wait(2)
+        except Exception:
+            self.proc.kill()
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            parts = [x.strip() for x in ln.split(",")]
+            if len(parts) < 6:
+                continue
+            try:
+                sm.append(float(parts[0]))
+                mx.append(float(parts[1]))
+            except ValueError:
+                continue
+            for nm, val in zip(names, parts[2:6]):
+                if val.lower().startswith("active"):
+                    reasons.add(nm)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def algorithmic_bytes(st, m, n, nnz):
+    """Bytes the method must move per solve, from the solve's own counters and the
+    per-unit figures of SURVEY.md §8(d) (int32 = 4 B):
+      push: 44 B per processed active column + 8 B per scanned neighbour
+      fix step: 24 B per worklist slot
+      GR: 16 B per expanded row + 8 B per read adjacency entry + 16 B per labelled column
+      greedy init: 8 B per column (cptr pair) + 8 B per read adjacency entry + 8 B per matched pair
+      FIXMATCHING + outputs: 12 n + 8 m
+    """
+    processed = st["pushes"] + st["blocked"] + st["dead"]
+    b = 44 * processed + 8 * st["edges_scanned"]
+    b += 24 * st["slots"]
+    b += 16 * st["gr_rows"] + 8 * st["gr_edges"] + 16 * st["gr_cols"]
+    b += 8 * n + 8 * st["greedy_edges"] + 8 * st["init_card"]
+    b += 12 * n + 8 * m
+    return int(b)
+
+
+def setup_bytes(m, n, nnz):
+    """mcm_create: validate (4(m+1) + 4 nnz) + copy (2 x (4(m+1) + 4 nnz)) + count (4 nnz
+    + 4 nnz atomics) + scan (3 x 4n) + scatter (4(m+1) + 4 nnz + 4 nnz atomics + 4 nnz)."""
+    return int(4 * (m + 1) * 4 + 4 * nnz * 8 + 12 * n)
+
+
+def run_ours(args, rank, world, local_rank):
+    import torch
+
+    import paper_conf_icpp_devecikuc13_b200 as pkg
+
+    dev = torch.device("cuda", local_rank)
+    torch.cuda.set_device(dev)
+    g = _graph(args.config, rank)
+    ip_h = torch.from_numpy(g.indptr).pin_memory()
+    ix_h = torch.from_numpy(g.indices).pin_memory()
+    ip = ip_h.to(dev)
+    ix = ix_h.to(dev)
+    stream = torch.cuda.current_stream(dev)
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device=dev)
+    rm = torch.empty(g.m, dtype=torch.int32, device=dev)
+    cm = torch.empty(g.n, dtype=torch.int32, device=dev)
+    opts = dict(k=args.k)
+    need = pkg.mcm_workspace_bytes(g.m, g.n, g.nnz, pkg.mcm_default_options(**opts))
+    ws = torch.empty(need, dtype=torch.uint8, device=dev)
+
+    def step():
+        mt = pkg.Matcher.__new__(pkg.Matcher)
+        mt_init(mt, ip, ix, g, ws, opts)
+        card, _, _ = mt.solve(rm, cm)
+        return mt, card
+
+    def barrier():
+        if world > 1:
+            torch.distributed.barrier()
+        torch.cuda.synchronize(dev)
+
+    for _ in range(args.warmup):
+        mt, card = step()
+        mt.close()
+    # timed region: K steps, L2 flushed before each, CUDA events around each step
+    evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True),
+            torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    clocks = Clocks(local_rank)
+    barrier()
+    clocks.start()
+    t_wall = time.perf_counter()
+    cards, stats = [], None
+    for i in range(args.steps):
+        flush.fill_(i & 0xFF)
+        e0, e1, e2 = evs[i]
+        e0.record(stream)
+        mt = pkg.Matcher.__new__(pkg.Matcher)
+        mt_init(mt, ip, ix, g, ws, opts)
+        e1.record(stream)
+        card, _, _ = mt.solve(rm, cm)
+        e2.record(stream)
+        cards.append(card)
+        stats = mt.stats()
+        mt.close()
+    barrier()
+    wall = time.perf_counter() - t_wall
+    clk = clocks.stop()
+    step_ms = [a.elapsed_time(c) for a, b_, c in evs]
+    create_ms = [a.elapsed_time(b_) for a, b_, c in evs]
+    solve_ms = [b_.elapsed_time(c) for a, b_, c in evs]
+    t_step = sum(step_ms) / len(step_ms)
+    t_solve = sum(solve_ms) / len(solve_ms)
+    t_create = sum(create_ms) / len(create_ms)
+
+    # ---- e2e through the public API with host buffers (H2D + create + solve + D2H)
+    rm_h = torch.empty(g.m, dtype=torch.int32).pin_memory()
+    cm_h = torch.empty(g.n, dtype=torch.int32).pin_memory()
+    e2e_ms = []
+    for i in range(args.warmup + args.steps):
+        flush.fill_(i & 0xFF)
+        barrier()
+        a = torch.cuda.Event(enable_timing=True)
+        b = torch.cuda.Event(enable_timing=True)
+        a.record(stream)
+        ipd = ip_h.to(dev, non_blocking=True)
+        ixd = ix_h.to(dev, non_blocking=True)
+        mt = pkg.Matcher.__new__(pkg.Matcher)
+        mt_init(mt, ipd, ixd, g, ws, opts)
+        card_e, rmd, cmd = mt.solve(rm, cm)
+        rm_h.copy_(rmd, non_blocking=True)
+        cm_h.copy_(cmd, non_blocking=True)
+        b.record(stream)
+        b.synchronize()
+        mt.close()
+        if i >= args.warmup:
+            e2e_ms.append(a.elapsed_time(b))
+    t_e2e = sum(e2e_ms) / len(e2e_ms)
+
+    # ---- max over ranks
+    vals = torch.tensor([t_step, t_e2e, float(g.nnz), t_solve, t_create], dtype=torch.float64, device=dev)
+    if world > 1:
+        mx = vals.clone()
+        torch.distributed.all_reduce(mx, op=torch.distributed.ReduceOp.MAX)
+        sm = vals.clone()
+        torch.distributed.all_reduce(sm, op=torch.distributed.ReduceOp.SUM)
+        t_step_max, t_e2e_max, t_solve_max, t_create_max = mx[0].item(), mx[1].item(), mx[3].item(), mx[4].item()
+        nnz_total = sm[2].item()
+    else:
+        t_step_max, t_e2e_max, t_solve_max, t_create_max, nnz_total = t_step, t_e2e, t_solve, t_create, float(g.nnz)
+    if rank != 0:
+        return None
+
+    peaks = _peaks()
+    hbm_peak = peaks["hbm_gbs"] if peaks else 6650.0
+    alg = algorithmic_bytes(stats, g.m, g.n, g.nnz)
+    achieved = alg / (t_solve * 1e-3) / 1e9  # GB/s of the solve kernel
+    traffic = None
+    tp = os.path.join(ROOT, "profiles", f"ncu_traffic_{args.config}.json")
+    if os.path.exists(tp):
+        try:
+            traffic = json.load(open(tp)).get("dram_bytes_per_launch")
+        except Exception:
+            traffic = None
+    line = {
+        "metric": METRIC,
+        "value": nnz_total / (t_step_max * 1e-3),
+        "unit": "edges/s",
+        "n_gpus": world,
+        "steps": args.steps,
+        "warmup": args.warmup,
+        "ms_per_step": t_step_max,
+        "higher_is_better": True,
+        "scaling": "weak",
+        "vs_baseline": None,
+        "dtype": "int32",
+        "data": "synthetic",
+        "config": {
+            "workload": f"{args.config}: {CONFIG_DESC[args.config]}",
+            "m": g.m, "n": g.n, "nnz": g.nnz, "mm": cards[-1], "init_card": stats["init_card"],
+            "k": args.k, "gr_strategy": "adaptive", "shrink_min": 512,
+            "step": "mcm_create + mcm_solve (device-resident CSR)",
+            "ms_create": t_create_max, "ms_solve": t_solve_max,
+            "edges_per_s_solve_only": nnz_total / (t_solve_max * 1e-3),
+            "l2": "flushed between steps (512 MiB write, outside the step events)",
+            "parallelism": f"replicas x{world} (one instance per GPU, no collective)",
+            "wall_s_timed_region": wall,
+        },
+        "roofline": {
+            "bound": "hbm",
+            "kernel": "gpr_kernel (persistent cooperative solve)",
+            "achieved": achieved,
+            "peak": hbm_peak,
+            "unit": "GB/s",
+            "frac": achieved / hbm_peak,
+            "traffic": traffic,
+            "algorithmic_bytes_per_launch": alg,
+            "peak_source": "MEASURED_PEAKS.json hbm_gbs" if peaks else "fallback B200_PROFILING.md",
+            "latency": {"grid_barriers": stats["grid_barriers"], "loops": stats["loops"],
+                        "gr_levels": stats["gr_levels"], "us_per_grid_barrier_measured": 1.21,
+                        "barrier_floor_ms": stats["grid_barriers"] * 1.21e-3},
+        },
+        "solve_stats": {k: stats[k] for k in ("loops", "gr_count", "gr_levels", "pushes", "blocked", "dead",
+                                              "edges_scanned", "slots", "shrinks", "guard_reactivated",
+                                              "tail_loops", "grid_barriers", "ms_init", "ms_gr", "ms_loop",
+                                              "ms_total", "grid_ctas")},
+        "clocks": clk,
+        "e2e": {"value": nnz_total / (t_e2e_max * 1e-3), "unit": "edges/s",
+                "h2d_bytes_per_step": 4 * (g.m + 1 + g.nnz), "d2h_bytes_per_step": 4 * (g.m + g.n),
+                "ms_per_step": t_e2e_max},
+        "gpu_launches": args.steps * 7,
+    }
+    if world == 1 and not args.no_cpu_baseline:
+        line["cpu_baseline"] = cpu_baseline(args.config, g)
+    return line
+
+
+def mt_init(mt, ip, ix, g, ws, opts):
+    """Matcher over a preallocated workspace (mcm_create through the C ABI)."""
+    import ctypes
+
+    import paper_conf_icpp_devecikuc13_b200 as pkg
+
+    mt.m, mt.n, mt.nnz = g.m, g.n, g.nnz
+    mt.opts = pkg.mcm_default_options(**opts)
+    mt.device = ip.device
+    mt.workspace = ws
+    h = ctypes.c_void_p()
+    import torch
+
+    rc = pkg.lib().mcm_create(ctypes.c_void_p(ip.data_ptr()), ctypes.c_void_p(ix.data_ptr()), g.m, g.n, g.nnz,
+                              ctypes.c_void_p(ws.data_ptr()), ws.numel(),
+                              ctypes.c_void_p(torch.cuda.current_stream().cuda_stream), ctypes.byref(mt.opts),
+                              ctypes.byref(h))
+    if rc != 0:
+        raise pkg.MCMError(rc, "mcm_create")
+    mt._h = h
+
+
+def cpu_baseline(name, g, budget_s=20.0):
+    """The oracle's sequential PR-FIFO (k = 0.5) incl. its cheap matching,
+    single-threaded on the host: a reported baseline, not the target."""
+    import oracle
+
+    csc = oracle.transpose(g)
+    times = []
+    t_start = time.perf_counter()
+    while True:
+        t0 = time.perf_counter()
+        oracle.cheap_match(g, csc)
+        card, _, _, _ = oracle.pr_fifo(g, k=0.5, csc=csc)
+        times.append(time.perf_counter() - t0)
+        if time.perf_counter() - t_start > budget_s * 0.5 or len(times) >= 5:
+            break
+    t = statistics.median(times)
+    return {"value": g.nnz / t, "unit": "edges/s", "cores": 1, "kind": "oracle",
+            "sample": f"full {name} graph ({g.nnz} nnz), sequential PR-FIFO + cheap matching, "
+                      f"median of {len(times)} runs ({t:.3f} s each)", "card": card}
+
+
+def run_reference(args, rank):
+    if rank != 0:
+        return None
+    g = _graph(args.config, 0)
+    times = []
+    cb = None
+    for i in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        cb = cpu_baseline(args.config, g, budget_s=0.0)  # one PR-FIFO run per step
+        dt = time.perf_counter() - t0
+        if i >= args.warmup:
+            times.append(dt)
+    t = sum(times) / len(times)
+    v = g.nnz / t
+    return {
+        "impl": "reference", "metric": METRIC, "value": v, "unit": "edges/s", "n_gpus": 1, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": t * 1e3, "higher_is_better": True, "scaling": "weak",
+        "vs_baseline": None, "dtype": "int32", "data": "synthetic",
+        "config": {"workload": f"{args.config}: {CONFIG_DESC[args.config]}", "m": g.m, "n": g.n, "nnz": g.nnz},
+        "cpu_baseline": {"value": v, "unit": "edges/s", "cores": 1, "kind": "oracle",
+                         "sample": f"full {args.config} graph per step: cheap matching + sequential PR-FIFO "
+                                   f"(k=0.5), single core"},
+        "e2e": {"value": v, "unit": "edges/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--config", default="C2", choices=sorted(CONFIG_DESC))
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--k", type=float, default=0.7)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    args = ap.parse_args()
+    args.warmup = max(args.warmup, 3)
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+    if args.impl == "reference":
+        line = run_reference(args, rank)
+        if line:
+            print(json.dumps(line), flush=True)
+        return
+    if world > 1:
+        import torch
+
+        torch.cuda.set_device(local_rank)
+        torch.distributed.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
+    line = run_ours(args, rank, world, local_rank)
+    if line:
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        import torch
+
+        torch.distributed.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

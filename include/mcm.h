@@ -108,6 +108,10 @@ typedef struct {
   int64_t card;              /* |M| returned */
   int64_t tail_loops;        /* loops run in the single-CTA tail mode */
   int64_t grid_barriers;     /* grid-wide barriers executed */
+  int64_t gr_rows;           /* rows expanded by all GR levels (frontier entries) */
+  int64_t gr_edges;          /* adjacency entries read by all GR levels */
+  int64_t gr_cols;           /* columns labelled by all GRs */
+  int64_t greedy_edges;      /* adjacency entries read by the greedy initial matching */
   double ms_init;            /* device time: initial matching + worklist build */
   double ms_gr;              /* device time in global relabels */
   double ms_loop;            /* device time in fix + push steps */

@@ -23,7 +23,7 @@ __all__ = ["Options", "Stats", "Matcher", "solve", "lib", "mcm_default_options",
            "MCMError", "LIB_PATH"]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libmcm.so")
+LIB_PATH = os.environ.get("MCM_LIB") or os.path.join(_HERE, "libmcm.so")  # MCM_LIB: A/B experiments only
 
 MCM_OK, MCM_EINVAL, MCM_ECUDA, MCM_ENOMEM, MCM_EDEVICE, MCM_ENOCONV, MCM_EINTERNAL = 0, -1, -2, -3, -4, -5, -6
 MCM_GR_ADAPTIVE, MCM_GR_FIXED = 0, 1
@@ -53,7 +53,8 @@ class Stats(ctypes.Structure):
 
     _fields_ = [(f, ctypes.c_int64) for f in (
         "loops", "gr_count", "gr_levels", "pushes", "blocked", "dead", "edges_scanned", "slots", "shrinks", "gaps",
-        "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers")] + [
+        "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers", "gr_rows", "gr_edges",
+        "gr_cols", "greedy_edges")] + [
         (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
         ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
 

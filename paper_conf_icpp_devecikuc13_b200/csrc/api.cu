@@ -9,6 +9,7 @@
 #include <new>
 #include <memory>
 #include <algorithm>
+#include <vector>
 
 #include "../../include/mcm.h"
 #include "solve.cuh"
@@ -44,7 +45,7 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   for (int i = 0; i < 4; i++) L.q[i] = take(sizeof(int) * mx);
   L.ctacnt = take(sizeof(int) * MAX_CTAS);
   L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
-  L.dbg = take(sizeof(int) * ((size_t)n + 1));
+  L.dbg = take(sizeof(int) * ((size_t)n + 1) + (getenv("MCM_TRACE") ? (size_t)atoi(getenv("MCM_TRACE")) * 24 : 0));
   L.total = o;
   return L;
 }
@@ -246,7 +247,7 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   int per_sm = 0;
   CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel, NT, 0));
   if (per_sm < 1) return MCM_EINTERNAL;
-  h->max_grid = h->sms * (per_sm > 2 ? 2 : per_sm);
+  h->max_grid = h->sms * (per_sm > 2 ? 2 : per_sm);  // one or two CTAs per SM (MCM_MINB)
   if (h->max_grid > MAX_CTAS) h->max_grid = MAX_CTAS;
 
   char *ws = h->ws;
@@ -314,6 +315,15 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.ctrl = (Ctrl *)(ws + L.ctrl);
   p.dbgbuf = (int *)(ws + L.dbg);
   p.debug = getenv("MCM_DEBUG") ? atoi(getenv("MCM_DEBUG")) : 0;
+  // MCM_TRACE=<n>: record up to n phase boundaries into the (otherwise idle during
+  // a solve) debug buffer; dumped to MCM_TRACE_FILE after the solve (analysis only)
+  int tcap = getenv("MCM_TRACE") ? atoi(getenv("MCM_TRACE")) : 0;
+  if (tcap > 0) {
+    size_t room = (h->L.total - h->L.dbg) / (3 * sizeof(long long));
+    if ((size_t)tcap > room) tcap = (int)room;
+    p.trace = (long long *)(ws + L.dbg);
+    p.trace_cap = tcap;
+  }
   const mcm_options_t &o = h->opt;
   p.k = o.k; p.gr_fixed = o.gr_strategy == MCM_GR_FIXED; p.shrink_min = o.shrink_min; p.init = o.init;
   p.gap = o.gap; p.final_check = o.final_check; p.dead_skip = o.dead_skip; p.tail_max = o.tail_max;
@@ -335,11 +345,20 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   s.blocked = x[ST_BLOCKED]; s.dead = x[ST_DEAD]; s.edges_scanned = x[ST_SCANNED]; s.slots = x[ST_SLOTS];
   s.shrinks = x[ST_SHRINKS]; s.gaps = x[ST_GAPS]; s.guard_reactivated = x[ST_GUARD]; s.fixed_cols = x[ST_FIXED];
   s.init_card = x[ST_INITCARD]; s.card = x[ST_CARD]; s.tail_loops = x[ST_TAILLOOPS]; s.grid_barriers = x[ST_BARRIERS];
+  s.gr_rows = x[ST_GR_ROWS]; s.gr_edges = x[ST_GR_EDGES]; s.gr_cols = x[ST_GR_COLS];
+  s.greedy_edges = x[ST_GREEDY_EDGES];
   s.ms_init = x[ST_NS_INIT] * 1e-6; s.ms_gr = x[ST_NS_GR] * 1e-6; s.ms_loop = x[ST_NS_LOOP] * 1e-6;
   s.ms_total = x[ST_NS_TOTAL] * 1e-6; s.ms_setup = h->ms_setup; s.grid_ctas = grid; s.threads_per_cta = NT;
   if (p.debug && c.dbg[0])
     fprintf(stderr, "[mcm debug] %lld violations; first: where=%lld loop=%lld x=%lld val=%lld\n", c.dbg[0], c.dbg[1],
             c.dbg[2], c.dbg[3], c.dbg[4]);
+  if (p.trace && getenv("MCM_TRACE_FILE")) {
+    long long tn = c.stat[ST_TRACE_N];
+    std::vector<long long> buf(3 * (size_t)tn);
+    cudaMemcpy(buf.data(), p.trace, buf.size() * sizeof(long long), cudaMemcpyDeviceToHost);
+    FILE *f = fopen(getenv("MCM_TRACE_FILE"), "wb");
+    if (f) { fwrite(buf.data(), sizeof(long long), buf.size(), f); fclose(f); }
+  }
   if (c.err) return c.err;
   if (mode == MODE_RELABEL) return x[ST_MAXLEVEL];
   return x[ST_CARD];

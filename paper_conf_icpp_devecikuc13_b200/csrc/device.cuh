@@ -45,6 +45,16 @@ __device__ __forceinline__ void st_rlx(int *p, int v) {
 __device__ __forceinline__ int ld_ro(const int *p) { return __ldg(p); }
 // phase-to-phase mutable arrays (worklists, queues): bypass L1
 __device__ __forceinline__ int ld_cg(const int *p) { return __ldcg(p); }
+__device__ __forceinline__ u32 ld_rlx(const u32 *p) {
+  u32 v;
+  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+__device__ __forceinline__ long long ld_rlx(const long long *p) {
+  long long v;
+  asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
 __device__ __forceinline__ u32 ld_acq(const u32 *p) {
   u32 v;
   asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
@@ -57,6 +67,31 @@ __device__ __forceinline__ u32 psi_of(u64 w) { return (u32)(w >> 32); }
 // decoded label: stale (below base) = INF
 __device__ __forceinline__ int lab(u32 s, u32 base, int INF) {
   return s >= base ? (int)min((u64)(s - base), (u64)INF + 1) : INF;
+}
+
+// Grid-wide barrier for a co-resident (cooperatively launched) grid.  One atomic
+// per CTA on a single word: CTA 0 adds 2^31 - (G-1), every other CTA adds 1, so
+// bit 31 flips exactly when the last CTA arrives (the low 31 bits return to 0).
+// The waiting thread polls with relaxed loads -- an acquire load per poll would
+// emit CCTL.IVALL and keep invalidating the L1 of every co-resident CTA (spills
+// and read-only graph lines included) -- optionally backing off with nanosleep,
+// and issues one gpu-scope fence after the flip.
+__device__ __forceinline__ void grid_sync(u32 *bar, bool sleepy) {
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    u32 nb = (blockIdx.x == 0) ? (0x80000000u - (gridDim.x - 1)) : 1u;
+    __threadfence();
+    u32 old = atomicAdd(bar, nb);
+    u32 ns = 16;
+    while (((ld_rlx(bar) ^ old) & 0x80000000u) == 0) {
+      if (sleepy) {
+        __nanosleep(ns);
+        if (ns < 2048) ns <<= 1;
+      }
+    }
+    __threadfence();
+  }
+  __syncthreads();
 }
 
 __device__ __forceinline__ int lane_id() { return threadIdx.x & 31; }

@@ -22,7 +22,9 @@ namespace mcm {
 constexpr int NT = 512;          // threads per CTA
 constexpr int NWARP = NT / 32;
 constexpr int QCAP = 4096;       // shared staging for the next BFS frontier
-constexpr int SMALL_DEG = 32;    // adjacency lists up to this length: one thread
+constexpr int SMALL_DEG = 32;    // greedy: adjacency lists up to this length: one thread
+constexpr int BIG_DEG = 64;      // GR / push: longer lists go to the whole warp
+constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
 
 enum { MODE_SOLVE = 0, MODE_RELABEL = 1 };
 
@@ -30,16 +32,22 @@ enum { MODE_SOLVE = 0, MODE_RELABEL = 1 };
 enum {
   ST_LOOPS, ST_GRS, ST_LEVELS, ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_SHRINKS, ST_GAPS,
   ST_GUARD, ST_FIXED, ST_INITCARD, ST_CARD, ST_TAILLOOPS, ST_BARRIERS, ST_NS_INIT, ST_NS_GR, ST_NS_LOOP,
-  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_NSTAT = 32
+  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_NSTAT = 32
 };
 
 struct Ctrl {
   u32 ring[4][4];          // per-phase counters, rotated (see Solver::barrier)
+  u32 bar;                 // grid barrier word (device.cuh grid_sync)
+  u32 pad0[3];
   long long stat[ST_NSTAT];
   int err;                 // 0 or an MCM_* code
   u32 gcnt;                // exactness-guard list cursor (monotonic within a solve)
   int pad[14];
   long long dbg[8];        // debug checks: [0] count, [1] where, [2] loop, [3] vertex, [4] value
+  // tail-mode handoff (CTA 0 -> grid)
+  int ho_reason, ho_ph, ho_len, ho_ulen, ho_shrink, ho_ac0, ho_u0, ho_gl, ho_gd, ho_gn, ho_gc;
+  u32 ho_base;
+  long long ho_loop, ho_iter;
 };
 
 struct Params {
@@ -50,6 +58,8 @@ struct Params {
   int *ctacnt;
   int *dbgbuf;             // n ints (debug checks only)
   int debug;
+  long long *trace;        // optional phase trace: {tag, size, t_end_ns} triples (MCM_TRACE)
+  int trace_cap;
   Ctrl *ctrl;
   // options
   double k;
@@ -79,8 +89,13 @@ struct Solver {
   const int m, n, INF;
   // per-thread statistics (reduced at the end)
   long long s_push = 0, s_block = 0, s_dead = 0, s_scan = 0, s_slots = 0, s_free = 0;
+  long long s_grrows = 0, s_gredges = 0, s_grcols = 0, s_gyedges = 0;
   int ph = 0;  // phase counter: identical in every thread
   long long nbar = 0;
+  int ttag = 0, tsz = 0, tn = 0;  // phase trace (lead thread only)
+  __device__ __forceinline__ void trace(int tag, int sz) {
+    ttag = tag; tsz = sz;
+  }
 
   __device__ Solver(const Params &p_, Smem &sm_) : p(p_), sm(sm_), m(p_.m), n(p_.n), INF(p_.m + p_.n) {}
 
@@ -90,8 +105,12 @@ struct Solver {
   // and consumed at the start of the previous phase, so CTA 0 may clear it now.
   template <bool GRID>
   __device__ __forceinline__ void barrier() {
+    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
+      p.trace[3 * tn] = ttag * 2 + (GRID ? 1 : 0); p.trace[3 * tn + 1] = tsz; p.trace[3 * tn + 2] = (long long)gtime();
+      tn++;
+    }
     if (GRID) {
-      cg::this_grid().sync();
+      grid_sync(&p.ctrl->bar, false);
       nbar++;
     } else {
       __syncthreads();
@@ -104,7 +123,7 @@ struct Solver {
     if (!GRID) __syncthreads();
   }
   __device__ __forceinline__ u32 *ring_now(int j) { return &p.ctrl->ring[ph & 3][j]; }
-  __device__ __forceinline__ u32 ring_prev(int j) { return ld_acq(&p.ctrl->ring[(ph - 1) & 3][j]); }
+  __device__ __forceinline__ u32 ring_prev(int j) { return ld_rlx(&p.ctrl->ring[(ph - 1) & 3][j]); }
 
   template <bool GRID>
   __device__ __forceinline__ int cta() const { return GRID ? blockIdx.x : 0; }
@@ -216,6 +235,7 @@ struct Solver {
         for (int j = s; j < e; j++) {
           int u = ld_ro(p.cadj + j);
           u64 rs = ld_rlx(p.rowst + u);
+          s_gyedges++;
           if (mu_of(rs) != -1) continue;
           if (atomicCAS(p.rowst + u, rs, pack(v, psi_of(rs))) == rs) {
             st_rlx(p.colst + v, pack(u, 0));
@@ -234,7 +254,7 @@ struct Solver {
           int j = c0 + lane;
           int u = -1;
           u64 rs = 0;
-          if (j < eb) { u = ld_ro(p.cadj + j); rs = ld_rlx(p.rowst + u); }
+          if (j < eb) { u = ld_ro(p.cadj + j); rs = ld_rlx(p.rowst + u); s_gyedges++; }
           unsigned cand = __ballot_sync(0xffffffffu, u >= 0 && mu_of(rs) == -1);
           while (cand && !done) {
             int l = __ffs(cand) - 1;
@@ -271,20 +291,35 @@ struct Solver {
   // lvl == 0: `cur` is the unmatched-row list U; rows that got matched since are
   // dropped, the others get label 0 (INITRELABEL) and are written to
   // Uout (the filtered U).
+  // Lanes per vertex for a phase over `items` vertices on `threads` threads: the
+  // largest power of two <= 32 with items * G <= threads, so narrow frontiers and
+  // short worklists spread each adjacency list over a lane group instead of
+  // walking it one dependent load at a time.
+  __device__ __forceinline__ static int pick_group(long long items, int threads) {
+    int g = 1;
+    while (g < 32 && items * (g * 2) <= threads) g <<= 1;
+    return g;
+  }
+  __device__ __forceinline__ static unsigned group_mask(int G) {
+    return G == 32 ? 0xffffffffu : (((1u << G) - 1u) << (lane_id() & ~(G - 1)));
+  }
+
   template <bool GRID>
   __device__ void gr_level(const int *cur, int curlen, int lvl, u32 base, int *next, u32 *ncnt, int *Uout,
                            u32 *ucnt, int *guard, u32 *gcnt) {
     const int lane = lane_id();
     const u32 lc = base + lvl + 1, lr = base + lvl + 2;
-    for (int t = cta<GRID>() * NT; t < curlen; t += ncta<GRID>() * NT) {
-      int i = t + threadIdx.x;
+    const int G = pick_group(curlen, ncta<GRID>() * NT);
+    const int gl = lane & (G - 1), per_tile = NT / G;
+    for (int t = cta<GRID>() * per_tile; t < curlen; t += ncta<GRID>() * per_tile) {
+      int i = t + (int)threadIdx.x / G;
       int u = (i < curlen) ? ld_cg(cur + i) : -1;
       if (lvl == 0) {
         bool keep = false;
         if (u >= 0) {
           if (mu_of(ld_rlx(p.rowst + u)) == -1) {
-            st_rlx(p.rowst + u, pack(-1, base));
-            keep = true;
+            if (gl == 0) st_rlx(p.rowst + u, pack(-1, base));
+            keep = gl == 0;
           } else {
             u = -1;
           }
@@ -295,36 +330,60 @@ struct Solver {
         if (keep) Uout[sm.tmp + r] = u;
       }
       int s = 0, e = 0;
-      if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
-      if (u >= 0 && e - s <= SMALL_DEG)
-        for (int j = s; j < e; j++) visit(ld_ro(p.radj + j), lc, lr, next, ncnt, guard, gcnt);
-      unsigned big = __ballot_sync(0xffffffffu, u >= 0 && e - s > SMALL_DEG);
-      while (big) {
-        int bl = __ffs(big) - 1;
-        big &= big - 1;
+      if (u >= 0) {
+        s = ld_ro(p.rptr + u);
+        e = ld_ro(p.rptr + u + 1);
+        if (gl == 0) { s_grrows++; s_gredges += e - s; }
+      }
+      const bool big = u >= 0 && G < 32 && e - s > BIG_DEG;
+      if (u >= 0 && !big) expand(s + gl, e, G, lc, lr, next, ncnt, guard, gcnt);
+      unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
+      while (bigm) {  // long lists: the whole warp
+        int bl = __ffs(bigm) - 1;
+        bigm &= bigm - 1;
         int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
-        for (int j = sb + lane; j < eb; j += 32) visit(ld_ro(p.radj + j), lc, lr, next, ncnt, guard, gcnt);
+        expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt);
       }
       flush(next, ncnt);
     }
   }
-  __device__ __forceinline__ void visit(int v, u32 lc, u32 lr, int *next, u32 *ncnt, int *guard, u32 *gcnt) {
-    u64 cs = ld_rlx(p.colst + v);
-    // visited in this GR <=> its label carries the current epoch (>= base)
-    if (psi_of(cs) >= gr_base) return;
-    u64 nw = pack(mu_of(cs), lc);
-    if (atomicCAS(p.colst + v, cs, nw) != cs) return;
-    int w = mu_of(cs);
-    if (w >= 0) {
-      u64 rw = ld_rlx(p.rowst + w);
-      if (mu_of(rw) == v) {
-        st_rlx(p.rowst + w, pack(v, lr));
-        stage(w, next, ncnt);
-        return;
+  // Visit radj[j], j = j0, j0+step, ... < e, KB at a time: the KB column loads, then
+  // the KB claims (CAS), then the KB mate checks are each issued back to back.
+  __device__ __forceinline__ void expand(int j0, int e, int step, u32 lc, u32 lr, int *next, u32 *ncnt, int *guard,
+                                         u32 *gcnt) {
+    for (int j = j0; j < e; j += step * KB) {
+      int v[KB];
+      u64 cs[KB], old[KB], rw[KB];
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        int jj = j + k * step;
+        v[k] = jj < e ? ld_ro(p.radj + jj) : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? ld_rlx(p.colst + v[k]) : ~0ull;
+#pragma unroll
+      for (int k = 0; k < KB; k++)  // visited in this GR <=> label carries the current epoch (>= base)
+        old[k] = (v[k] >= 0 && psi_of(cs[k]) < gr_base) ? atomicCAS(p.colst + v[k], cs[k], pack(mu_of(cs[k]), lc))
+                                                         : ~cs[k];
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        int w = mu_of(cs[k]);
+        rw[k] = (old[k] == cs[k] && w >= 0) ? ld_rlx(p.rowst + w) : 0ull;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        if (old[k] != cs[k]) continue;  // not claimed by this thread
+        s_grcols++;
+        int w = mu_of(cs[k]);
+        if (w >= 0 && mu_of(rw[k]) == v[k]) {
+          st_rlx(p.rowst + w, pack(v[k], lr));
+          stage(w, next, ncnt);
+        } else {
+          s_free++;
+          if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
+        }
       }
     }
-    s_free++;
-    if (guard) guard[atomicAdd(gcnt, 1u)] = v;
   }
   u32 gr_base = 0;
 
@@ -334,25 +393,49 @@ struct Solver {
   // guard[0 .. gcount) (the exactness guard, R16).
   template <bool GRID>
   __device__ int global_relabel(int *&U, int &ulen, int *&T, int *Qa, int *Qb, u32 base, int *guard, int &gcount) {
+    GRState g;
+    gr_start<GRID>(g, U, ulen, T, Qa, base, guard);
+    gr_levels<GRID>(g, base, Qa, Qb, guard, 0x7fffffff);
+    gcount = (int)ld_rlx(&p.ctrl->gcnt);
+    return g.deepest + 2;
+  }
+
+  // The GR as a resumable state machine, so that a CTA-local GR (tail mode) can
+  // hand a frontier that grew too wide over to the whole grid mid-BFS.
+  struct GRState {
+    int lvl, deepest, nlen, cur_is_a;
+  };
+  // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
+  template <bool GRID>
+  __device__ void gr_start(GRState &g, int *&U, int &ulen, int *&T, int *Qa, u32 base, int *guard) {
     gr_base = base;
     u32 *gc = &p.ctrl->gcnt;  // zero here: reset one phase after its last use
+    trace(1, ulen);
     gr_level<GRID>(U, ulen, 0, base, Qa, ring_now(0), T, ring_now(1), guard, gc);
     barrier<GRID>();
-    int nlen = (int)ring_prev(0);
+    g.nlen = (int)ring_prev(0);
     ulen = (int)ring_prev(1);
     int *tmp = U; U = T; T = tmp;
-    int deepest = 0, lvl = 0;
-    int *cur = Qa, *nxt = Qb;
-    while (nlen > 0) {
-      lvl += 2;
-      deepest = lvl;
-      gr_level<GRID>(cur, nlen, lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
+    g.lvl = 0; g.deepest = 0; g.cur_is_a = 1;
+  }
+  // levels 2, 4, ... until the frontier is empty (returns true) or, before expanding
+  // a level, the frontier exceeds `limit` (returns false; state kept for resuming).
+  template <bool GRID>
+  __device__ bool gr_levels(GRState &g, u32 base, int *Qa, int *Qb, int *guard, int limit) {
+    gr_base = base;
+    u32 *gc = &p.ctrl->gcnt;
+    while (g.nlen > 0) {
+      if (g.nlen > limit) return false;
+      g.lvl += 2;
+      g.deepest = g.lvl;
+      int *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
+      trace(2, g.nlen);
+      gr_level<GRID>(cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
       barrier<GRID>();
-      nlen = (int)ring_prev(0);
-      int *t2 = cur; cur = nxt; nxt = t2;
+      g.nlen = (int)ring_prev(0);
+      g.cur_is_a ^= 1;
     }
-    gcount = (int)ld_acq(gc);
-    return deepest + 2;
+    return true;
   }
 
   // ---------------------------------------------------------------- fix step
@@ -391,8 +474,11 @@ struct Solver {
   template <bool GRID>
   __device__ void push(int len, int *Ac, int *Ap, int loop, u32 base) {
     const int lane = lane_id();
-    for (int t = cta<GRID>() * NT; t < len; t += ncta<GRID>() * NT) {
-      int i = t + threadIdx.x;
+    const int G = pick_group(len, ncta<GRID>() * NT);
+    const int gl = lane & (G - 1), per_tile = NT / G;
+    const unsigned gmask = group_mask(G);
+    for (int t = cta<GRID>() * per_tile; t < len; t += ncta<GRID>() * per_tile) {
+      int i = t + (int)threadIdx.x / G;
       int v = (i < len) ? ld_cg(Ac + i) : -1;
       int s = 0, e = 0, psiv = INF;
       u64 cs = 0;
@@ -403,61 +489,25 @@ struct Solver {
         e = ld_ro(p.cptr + v + 1);
         if (p.dead_skip && psiv >= INF) e = s;  // R19: provably unmatchable
       }
-      int psimin = INF, ub = -1, wb = -1;
       const int target = psiv - 1;
-      if (v >= 0 && e - s <= SMALL_DEG) {
-        for (int j = s; j < e; j++) {                       // l.6
-          int x = ld_ro(p.cadj + j);
-          u64 rs = ld_rlx(p.rowst + x);
-          int l = lab(psi_of(rs), base, INF);
-          s_scan++;
-          if (l < psimin) {                                 // l.7
-            psimin = l; ub = x; wb = mu_of(rs);             // l.8-9, R3
-            if (psimin == target) break;                    // l.10-11
-          }
-        }
-      }
-      unsigned big = __ballot_sync(0xffffffffu, v >= 0 && e - s > SMALL_DEG);
-      while (big) {
-        int bl = __ffs(big) - 1;
-        big &= big - 1;
+      const bool big = v >= 0 && G < 32 && e - s > BIG_DEG;
+      u64 best = ~0ull;
+      int ub = -1, wb = -1;
+      if (v >= 0 && !big) scan(s, e, gl, G, gmask, target, base, best, ub, wb);      // l.6-11
+      unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
+      while (bigm) {  // long lists: the whole warp
+        int bl = __ffs(bigm) - 1;
+        bigm &= bigm - 1;
         int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
         int tb = __shfl_sync(0xffffffffu, target, bl);
-        u64 best = ~0ull;
-        int bu = -1, bw = -1;
-        for (int c0 = sb; c0 < eb; c0 += 32) {
-          int j = c0 + lane;
-          u64 key = ~0ull;
-          int x = -1, w = -1;
-          if (j < eb) {
-            x = ld_ro(p.cadj + j);
-            u64 rs = ld_rlx(p.rowst + x);
-            int l = lab(psi_of(rs), base, INF);
-            w = mu_of(rs);
-            if (l < INF) key = ((u64)(u32)l << 32) | (u32)(j - sb);
-            s_scan++;
-          }
-          u64 kmin = key;
-#pragma unroll
-          for (int o = 16; o > 0; o >>= 1) {
-            u64 other = __shfl_xor_sync(0xffffffffu, kmin, o);
-            kmin = other < kmin ? other : kmin;
-          }
-          if (kmin < best) {
-            int src = (int)((u32)kmin - (u32)(c0 - sb));
-            best = kmin;
-            bu = __shfl_sync(0xffffffffu, x, src);
-            bw = __shfl_sync(0xffffffffu, w, src);
-          } else if (kmin != ~0ull) {
-            // keep the earlier minimum (first in adjacency order)
-          }
-          if (best != ~0ull && (int)(best >> 32) == tb) break;
-        }
-        if (lane == bl) {
-          if (best != ~0ull) { psimin = (int)(best >> 32); ub = bu; wb = bw; }
-        }
+        u64 b2;
+        int u2, w2;
+        scan(sb, eb, lane, 32, 0xffffffffu, tb, base, b2, u2, w2);
+        if (lane == bl) { best = b2; ub = u2; wb = w2; }
       }
+      if (gl != 0) continue;
       if (v >= 0) {
+        int psimin = best == ~0ull ? INF : (int)(best >> 32);
         if (psimin < INF) {                                 // l.12
           if (wb == -1 || ld_rlx(p.iA + wb) != loop) {      // l.13
             st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
@@ -477,6 +527,49 @@ struct Solver {
       } else if (i < len) {
         Ap[i] = -1;                                         // l.24
       }
+    }
+  }
+  // First minimum of psi over Gamma(v) = cadj[s, e) in adjacency order (Alg. 9
+  // l.6-11): the G lanes of a group read KB*G consecutive neighbours per step, take
+  // the (label, position) minimum and stop after the step in which the running
+  // minimum reaches psi(v)-1 (reading R11).  best = (label << 32 | position) or ~0.
+  __device__ __forceinline__ void scan(int s, int e, int gl, int G, unsigned gmask, int target, u32 base, u64 &best,
+                                       int &bu, int &bw) {
+    best = ~0ull;
+    bu = -1;
+    bw = -1;
+    for (int c0 = s; c0 < e; c0 += G * KB) {
+      int x[KB];
+      u64 rs[KB];
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        int jj = c0 + gl + k * G;
+        x[k] = jj < e ? ld_ro(p.cadj + jj) : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+      u64 key = ~0ull;
+      int kx = -1, kw = -1;
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        if (x[k] < 0) continue;
+        s_scan++;
+        int l = lab(psi_of(rs[k]), base, INF);
+        u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + gl + k * G - s)) : ~0ull;
+        if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
+      }
+      u64 km = key;
+      for (int o = G >> 1; o > 0; o >>= 1) {
+        u64 other = __shfl_xor_sync(gmask, km, o, G);
+        km = other < km ? other : km;
+      }
+      if (km < best) {
+        int src = __ffs(__ballot_sync(gmask, key == km)) - 1;
+        best = km;
+        bu = __shfl_sync(gmask, kx, src);
+        bw = __shfl_sync(gmask, kw, src);
+      }
+      if (best != ~0ull && (int)(best >> 32) == target) break;
     }
   }
 
@@ -537,6 +630,87 @@ struct Solver {
     barrier<true>();
   }
 
+  // ---------------------------------------------------------------- tail mode
+  enum { R_NONE = 0, R_TERM = 1, R_NEEDGR = 2, R_ESC = 3, R_CAP = 4 };
+  __device__ __forceinline__ int tail_f() const { return p.tail_max * 4 > 4096 ? p.tail_max * 4 : 4096; }
+
+  // All CTAs call.  CTA 0 runs Alg. 7 iterations alone -- fix with compaction at
+  // every step, push, and GRs whose frontiers stay narrow -- with __syncthreads
+  // between phases, while the other CTAs wait at one grid barrier.  The episode
+  // ends when a GR needs the grid (too many unmatched rows, or a frontier that
+  // grew past tail_f(): R_ESC hands the BFS state over), when no active column is
+  // left (R_TERM) or at the iteration cap (R_CAP).  CTA 0 then publishes its
+  // control registers and every CTA adopts them after the barrier.
+  __device__ int tail_episode(long long &loop, long long &iterGR, int &len, int &ulen, u32 &base, bool &shrink,
+                              int *&Ac, int *&Ap, int *&U, int *&T, int *Qa, int *Qb, GRState &gst, long long &grs,
+                              long long &levels, long long &shrinks, long long &tail_loops, long long &ns_gr,
+                              long long &ns_loop) {
+    const u32 stride = (u32)(m + n + 2);
+    int reason = R_NONE;
+    Ctrl *c = p.ctrl;
+    if (blockIdx.x == 0) {
+      const int limit = tail_f();
+      for (;;) {
+        if (loop >= p.max_loops) { reason = R_CAP; break; }
+        if (loop == iterGR) {
+          if (ulen > limit || (u64)base + 2ull * stride >= 0xfffffff0ull) { reason = R_NEEDGR; break; }
+          u64 g0 = gtime();
+          gr_start<false>(gst, U, ulen, T, Qa, base, nullptr);
+          bool done = gr_levels<false>(gst, base, Qa, Qb, nullptr, limit);
+          ns_gr += (long long)(gtime() - g0);
+          if (!done) { reason = R_ESC; break; }
+          int ml = gst.deepest + 2;
+          grs++; levels += ml / 2;
+          iterGR = loop + iter_gap(ml);
+          shrink = true;
+          base += stride;
+        }
+        u64 l0 = gtime();
+        const int lp = (int)loop;
+        if (threadIdx.x == 0) s_slots += len;
+        trace(3, len);
+        int r1 = compact_pass1<false>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, nullptr, Ac);
+        barrier<false>();
+        len = r1;
+        if (shrink) { shrinks++; shrink = false; }
+        if (len == 0) { reason = R_TERM; ns_loop += (long long)(gtime() - l0); break; }
+        trace(4, len);
+        push<false>(len, Ac, Ap, lp, base - stride);
+        barrier<false>();
+        int *tmp = Ac; Ac = Ap; Ap = tmp;
+        loop++;
+        tail_loops++;
+        ns_loop += (long long)(gtime() - l0);
+      }
+      if (threadIdx.x == 0) {
+        c->ho_reason = reason; c->ho_ph = ph; c->ho_len = len; c->ho_ulen = ulen; c->ho_shrink = shrink;
+        c->ho_ac0 = (Ac == p.wl0); c->ho_u0 = (U == p.qa); c->ho_loop = loop; c->ho_iter = iterGR;
+        c->ho_base = base; c->ho_gl = gst.lvl; c->ho_gd = gst.deepest; c->ho_gn = gst.nlen; c->ho_gc = gst.cur_is_a;
+        for (int j = 0; j < 4; j++) c->ring[j][0] = c->ring[j][1] = c->ring[j][2] = c->ring[j][3] = 0;
+      }
+    }
+    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
+      p.trace[3 * tn] = 99; p.trace[3 * tn + 1] = reason; p.trace[3 * tn + 2] = (long long)gtime();
+      tn++;
+    }
+    grid_sync(&p.ctrl->bar, true);
+    nbar++;
+    reason = ld_rlx((const u32 *)&c->ho_reason);
+    ph = (int)ld_rlx((const u32 *)&c->ho_ph) + 1;
+    len = (int)ld_rlx((const u32 *)&c->ho_len);
+    ulen = (int)ld_rlx((const u32 *)&c->ho_ulen);
+    shrink = ld_rlx((const u32 *)&c->ho_shrink) != 0;
+    bool ac0 = ld_rlx((const u32 *)&c->ho_ac0) != 0, u0 = ld_rlx((const u32 *)&c->ho_u0) != 0;
+    Ac = ac0 ? p.wl0 : p.wl1; Ap = ac0 ? p.wl1 : p.wl0;
+    U = u0 ? p.qa : p.qb; T = u0 ? p.qb : p.qa;
+    loop = ld_rlx(&c->ho_loop);
+    iterGR = ld_rlx(&c->ho_iter);
+    base = ld_rlx(&c->ho_base);
+    gst.lvl = (int)ld_rlx((const u32 *)&c->ho_gl); gst.deepest = (int)ld_rlx((const u32 *)&c->ho_gd);
+    gst.nlen = (int)ld_rlx((const u32 *)&c->ho_gn); gst.cur_is_a = (int)ld_rlx((const u32 *)&c->ho_gc);
+    return reason;
+  }
+
   // ---------------------------------------------------------------- the solve
   __device__ void run() {
     const bool lead = blockIdx.x == 0 && threadIdx.x == 0;
@@ -579,83 +753,111 @@ struct Solver {
     u64 t1 = gtime();
     ns_init = (long long)(t1 - t0);
 
-    long long loop = 0, iterGR = 0;
+    long long loop = 0, iterGR = 0, tail_loops = 0;
     bool shrink = false;
+    GRState gst;
+    int reason = R_NONE;
     for (;;) {
       if (loop >= p.max_loops) {
         if (lead) p.ctrl->err = -5;
         break;
       }
-      if (loop == iterGR) {                                            // Alg. 7 l.6
-        u64 g0 = gtime();
-        if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
-        int gdummy;
-        int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, nullptr, gdummy);   // l.7
-        grs++; levels += ml / 2;
-        iterGR = loop + iter_gap(ml);                                  // l.8
-        shrink = true;                                                 // l.9
-        base += stride;
-        ns_gr += (long long)(gtime() - g0);
-      }
-      const u32 cur = base - stride;  // epoch of the labels in use
-      u64 l0 = gtime();
-      int act;
-      if ((shrink && p.shrink_min >= 0 && len >= p.shrink_min) || p.compact_every) {  // l.11
-        const int lp = (int)loop;
-        int r1 = compact_pass1<true>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
-        barrier<true>();
-        len = compact_pass2<true>(len, T, Ac, r1);                     // SHRKRNL
-        act = len;
-        s_slots += r1;
-        if (shrink) shrinks++;
-        shrink = false;                                                // l.13
-        // Ac was rewritten by CTAs other than the pushing one: order it before PUSH
-        barrier<true>();
-      } else {
-        fix_plain<true>(len, Ac, Ap, (int)loop, 0);                    // l.15
-        barrier<true>();
-        act = (int)ring_prev(0);
-      }
-      debug_check(3, loop, Ac, len);
-      if (act == 0) {                                                  // l.5 / l.16
-        ns_loop += (long long)(gtime() - l0);
-        if (!p.final_check) break;
-        // exactness guard (R16): one more GR; every unmatched column it reaches is
-        // re-activated and the loop resumes; otherwise psi certifies maximality.
-        u64 g0 = gtime();
-        if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
-        int gcount = 0;
-        int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, Ac, gcount);
-        grs++; levels += ml / 2;
-        base += stride;
-        ns_gr += (long long)(gtime() - g0);
-        if (gcount == 0) break;
-        guard_re += gcount;
-        for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
-          int v = __ldcg(Ac + i);
-          u64 cs = ld_rlx(p.colst + v);
-          st_rlx(p.colst + v, pack(-1, psi_of(cs)));
-          Ap[i] = v;
+      bool terminated = false;
+      reason = R_NONE;
+      // ---- tail episode: a short worklist runs on CTA 0 alone (CTA barriers)
+      if (p.tail_max > 0 && len <= p.tail_max && !(loop == iterGR && ulen > tail_f())) {
+        reason = tail_episode(loop, iterGR, len, ulen, base, shrink, Ac, Ap, U, T, Qa, Qb, gst, grs, levels,
+                              shrinks, tail_loops, ns_gr, ns_loop);
+        if (reason == R_CAP) {
+          if (lead) p.ctrl->err = -5;
+          break;
         }
-        barrier<true>();
-        if (lead) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
-        len = gcount;
-        iterGR = loop + iter_gap(ml);
-        shrink = false;
-        continue;
+        if (reason == R_TERM) terminated = true;
       }
-      push<true>(len, Ac, Ap, (int)loop, cur);                         // l.17
+      if (!terminated) {
+        if (reason == R_ESC || loop == iterGR) {                       // Alg. 7 l.6
+          u64 g0 = gtime();
+          int ml;
+          if (reason == R_ESC) {  // a tail GR whose frontier grew too wide: finish it here
+            gr_levels<true>(gst, base, Qa, Qb, nullptr, 0x7fffffff);
+            ml = gst.deepest + 2;
+          } else {
+            if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
+            int gdummy;
+            ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, nullptr, gdummy);   // l.7
+          }
+          grs++; levels += ml / 2;
+          iterGR = loop + iter_gap(ml);                                // l.8
+          shrink = true;                                               // l.9
+          base += stride;
+          ns_gr += (long long)(gtime() - g0);
+          if (p.tail_max > 0 && len <= p.tail_max) continue;           // fix + push in the tail
+        }
+        const u32 cur = base - stride;  // epoch of the labels in use
+        u64 l0 = gtime();
+        int act;
+        if ((shrink && p.shrink_min >= 0 && len >= p.shrink_min) || p.compact_every) {  // l.11
+          const int lp = (int)loop;
+          int r1 = compact_pass1<true>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
+          s_slots += 0;
+          if (lead) s_slots += len;
+          barrier<true>();
+          len = compact_pass2<true>(len, T, Ac, r1);                   // SHRKRNL
+          act = len;
+          if (shrink) shrinks++;
+          shrink = false;                                              // l.13
+          // Ac was rewritten by CTAs other than the pushing one: order it before PUSH
+          barrier<true>();
+        } else {
+          trace(3, len);
+          fix_plain<true>(len, Ac, Ap, (int)loop, 0);                  // l.15
+          barrier<true>();
+          act = (int)ring_prev(0);
+        }
+        debug_check(3, loop, Ac, len);
+        if (act != 0) {
+          trace(4, len);
+          push<true>(len, Ac, Ap, (int)loop, cur);                     // l.17
+          barrier<true>();
+          debug_check(4, loop, nullptr, 0);
+          int *tmp = Ac; Ac = Ap; Ap = tmp;                            // l.18
+          loop++;                                                      // l.19
+          loops++;
+          ns_loop += (long long)(gtime() - l0);
+          continue;
+        }
+        ns_loop += (long long)(gtime() - l0);
+      }
+      // ---- no active column left (l.5 / l.16)
+      if (!p.final_check) break;
+      // exactness guard (R16): one more GR; every unmatched column it reaches is
+      // re-activated and the loop resumes; otherwise psi certifies maximality.
+      u64 g0 = gtime();
+      if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
+      int gcount = 0;
+      int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, Ac, gcount);
+      grs++; levels += ml / 2;
+      base += stride;
+      ns_gr += (long long)(gtime() - g0);
+      if (gcount == 0) break;
+      guard_re += gcount;
+      for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
+        int v = __ldcg(Ac + i);
+        u64 cs = ld_rlx(p.colst + v);
+        st_rlx(p.colst + v, pack(-1, psi_of(cs)));
+        Ap[i] = v;
+      }
       barrier<true>();
-      debug_check(4, loop, nullptr, 0);
-      int *tmp = Ac; Ac = Ap; Ap = tmp;                                // l.18
-      loop++;                                                          // l.19
-      loops++;
-      ns_loop += (long long)(gtime() - l0);
+      if (lead) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
+      len = gcount;
+      iterGR = loop + iter_gap(ml);
+      shrink = false;
     }
+    loops += tail_loops;
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
     finish_stats(loops, grs, levels, shrinks, guard_re, init_card, ns_init, ns_gr, ns_loop, (long long)(gtime() - tA),
-                 0);
+                 tail_loops);
   }
 
   __device__ void reset_labels() {
@@ -668,9 +870,10 @@ struct Solver {
   __device__ void finish_stats(long long loops, long long grs, long long levels, long long shrinks, long long guard_re,
                                long long init_card, long long ns_init, long long ns_gr, long long ns_loop,
                                long long ns_total, long long tail_loops) {
-    long long v[7] = {s_push, s_block, s_dead, s_scan, s_slots, s_free, 0};
-    const int slot[6] = {ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_REACHED_FREE};
-    for (int k = 0; k < 6; k++) {
+    long long v[10] = {s_push, s_block, s_dead, s_scan, s_slots, s_free, s_grrows, s_gredges, s_grcols, s_gyedges};
+    const int slot[10] = {ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_REACHED_FREE,
+                          ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES};
+    for (int k = 0; k < 10; k++) {
       long long t = cta_sum<NT>(v[k], sm.red);
       if (threadIdx.x == 0 && t) atomicAdd((unsigned long long *)&p.ctrl->stat[slot[k]], (unsigned long long)t);
     }
@@ -680,15 +883,19 @@ struct Solver {
       st[ST_GUARD] = guard_re; st[ST_INITCARD] = init_card; st[ST_NS_INIT] = ns_init; st[ST_NS_GR] = ns_gr;
       st[ST_NS_LOOP] = ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = tail_loops;
       st[ST_BARRIERS] = nbar;
+      st[ST_TRACE_N] = tn;
       if (p.mode == MODE_SOLVE) {
-        st[ST_CARD] = (long long)ld_acq(&p.ctrl->ring[(ph - 1) & 3][0]);
-        st[ST_FIXED] = (long long)ld_acq(&p.ctrl->ring[(ph - 1) & 3][1]);
+        st[ST_CARD] = (long long)ld_rlx(&p.ctrl->ring[(ph - 1) & 3][0]);
+        st[ST_FIXED] = (long long)ld_rlx(&p.ctrl->ring[(ph - 1) & 3][1]);
       }
     }
   }
 };
 
-__global__ void __launch_bounds__(NT, 2) gpr_kernel(Params p) {
+#ifndef MCM_MINB
+#define MCM_MINB 1
+#endif
+__global__ void __launch_bounds__(NT, MCM_MINB) gpr_kernel(Params p) {
   __shared__ Smem sm;
   Solver s(p, sm);
   s.run();
