@@ -83,11 +83,16 @@ typedef struct {
                            any unmatched column it reaches is re-activated (R16). */
   int32_t dead_skip;    /* 1 (default): an active column whose label is already
                            >= m+n dies without scanning Gamma(v) (R19). */
-  int32_t tail_max;     /* worklists of at most this many slots run on one CTA with
-                           CTA barriers instead of grid barriers (0 = off); default 2048 */
+  int32_t tail_max;     /* worklists of at most this many slots run on the tail group
+                           (tail_ctas CTAs) instead of the whole grid (0 = off); GRs whose
+                           frontiers stay within 2*tail_max rows too; default 4096 */
   int32_t compact_every;/* 1: compact the worklist at every fix step (an option beyond
                            the paper's post-GR shrink); default 0 */
   int32_t grid_ctas;    /* CTAs of the persistent kernel; 0 (default) = all co-resident */
+  int32_t tail_ctas;    /* CTAs of the tail group: 1 = one CTA (__syncthreads), 2..16 = a
+                           thread-block cluster (hardware cluster barrier); default 8 */
+  int32_t compact_adapt;/* 1 (default): compact the worklist at the next fix step when
+                           fewer than 1/4 of its slots hold an active column */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 
@@ -150,6 +155,15 @@ int64_t mcm_solve(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t 
  * are not matched but got a finite label (> 0 iff an augmenting path exists). */
 int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,
                            int32_t *psi_row, int32_t *psi_col, int64_t *reached_free);
+
+/* Gap relabelling (reading R14) of given labels, in place: psi_row (m)
+ * and psi_col (n) are DEVICE int32 labels (values >= m+n, or < 0, mean infinite).
+ * Counts the vertices of every finite label below H = min(m+n+2, 2^20); if some
+ * label g below the largest finite label has no vertex, every label in (g, m+n)
+ * becomes m+n (labels >= m+n are written back as m+n).  Returns g, or -1 when there
+ * is no gap, or a negative error code below -1.  This is the same device routine
+ * the solve applies once between two GRs when options.gap = 1. */
+int64_t mcm_gap_relabel(mcm_handle_t h, mcm_stream_t stream, int32_t *psi_row, int32_t *psi_col);
 
 /* Replace the options of a handle (takes effect at the next solve). */
 int mcm_set_options(mcm_handle_t h, const mcm_options_t *o);

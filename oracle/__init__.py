@@ -64,6 +64,8 @@ def _get():
         lib.or_konig_cover.restype = i64
         lib.or_gpr_serial.argtypes = [i32, i32, P32, P32, P32, P32, P32, P32, dbl, P64, P64]
         lib.or_gpr_serial.restype = i64
+        lib.or_gap_relabel.argtypes = [i32, i32, P32, P32, i32]
+        lib.or_gap_relabel.restype = ctypes.c_int
         _lib = lib
     return _lib
 
@@ -185,18 +187,30 @@ def konig_cover(g, rmatch, cmatch):
     return int(size), cr[: g.m], cc[: g.n]
 
 
+def gap_relabel(m, n, psi_row, psi_col, H=None):
+    """Reading R14 on copies of the labels -> (g, psi_row', psi_col'); g = -1: no gap."""
+    if H is None:
+        H = min(m + n + 2, 1 << 20)
+    pr = np.concatenate([_i32(psi_row), [0]]).astype(np.int32)
+    pc = np.concatenate([_i32(psi_col), [0]]).astype(np.int32)
+    gl = _get().or_gap_relabel(m, n, _p32(pr), _p32(pc), H)
+    if gl < -1:
+        raise RuntimeError(gl)
+    return int(gl), pr[:m], pc[:n]
+
+
 def gpr_serial(g, k: float = 0.7, gr_fixed: bool = False, shrink_min: int = 512, dead_skip: bool = False,
-               init="greedy", max_loops: int = 0, csc=None):
+               init="greedy", max_loops: int = 0, gap: bool = False, csc=None):
     """Serial G-PR (Alg. 7/8/9) -> (card, mu_row, mu_col, stats dict)."""
     csc = csc or transpose(g)
     rm, cm = _init(g, init, csc)
-    opts = np.array([int(gr_fixed), shrink_min, int(dead_skip), max_loops], np.int64)
-    st = np.zeros(7, np.int64)
+    opts = np.array([int(gr_fixed), shrink_min, int(dead_skip), max_loops, int(gap)], np.int64)
+    st = np.zeros(8, np.int64)
     card = _get().or_gpr_serial(g.m, g.n, _p32(g.indptr), _p32(_adj(g)), _p32(csc.cptr), _p32(csc.cadj),
                                 _p32(rm), _p32(cm), k, _p64(opts), _p64(st))
     if card < 0:
         raise RuntimeError(card)
-    keys = ["loops", "grs", "levels", "pushes", "shrinks", "dead", "blocked"]
+    keys = ["loops", "grs", "levels", "pushes", "shrinks", "dead", "blocked", "gaps"]
     return int(card), rm[: g.m], cm[: g.n], dict(zip(keys, map(int, st)))
 
 

@@ -44,6 +44,8 @@ class Options(ctypes.Structure):
         ("tail_max", ctypes.c_int32),
         ("compact_every", ctypes.c_int32),
         ("grid_ctas", ctypes.c_int32),
+        ("tail_ctas", ctypes.c_int32),
+        ("compact_adapt", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]
 
@@ -56,7 +58,9 @@ class Stats(ctypes.Structure):
         "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers", "gr_rows", "gr_edges",
         "gr_cols", "greedy_edges")] + [
         (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
-        ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
+        ("grid_ctas", ctypes.c_int32),
+        ("tail_ctas", ctypes.c_int32),
+        ("compact_adapt", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
 
     def as_dict(self):
         return {f: getattr(self, f) for f, _ in self._fields_}
@@ -90,6 +94,8 @@ def lib():
         L.mcm_solve.restype = i64
         L.mcm_global_relabel.argtypes = [vp, vp, vp, vp, vp, vp, P(i64)]
         L.mcm_global_relabel.restype = i64
+        L.mcm_gap_relabel.argtypes = [vp, vp, vp, vp]
+        L.mcm_gap_relabel.restype = i64
         L.mcm_set_options.argtypes = [vp, P(Options)]
         L.mcm_set_options.restype = ctypes.c_int
         L.mcm_set_k.argtypes = [vp, ctypes.c_double]
@@ -205,6 +211,18 @@ class Matcher:
         if ml < 0:
             raise MCMError(int(ml), "mcm_global_relabel")
         return int(ml), pr, pc, int(rf.value)
+
+    def gap_relabel(self, psi_row, psi_col, stream=None):
+        """mcm_gap_relabel on copies of the given labels -> (gap, psi_row', psi_col')."""
+        torch = _torch()
+        pr = psi_row.to(self.device, torch.int32).contiguous().clone()
+        pc = psi_col.to(self.device, torch.int32).contiguous().clone()
+        with torch.cuda.device(self.device):
+            g = lib().mcm_gap_relabel(self._h, _stream_ptr(stream), _dev_i32(pr, "psi_row", self.m),
+                                      _dev_i32(pc, "psi_col", self.n))
+        if g < -1:
+            raise MCMError(int(g), "mcm_gap_relabel")
+        return int(g), pr, pc
 
     def stats(self) -> dict:
         s = Stats()

@@ -24,7 +24,8 @@ constexpr int MAX_CTAS = 4096;
 size_t align256(size_t x) { return (x + 255) & ~(size_t)255; }
 
 struct Layout {
-  size_t ctrl, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, dbg, total;
+  size_t ctrl, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, dbg, total;
+  int hist_len;
 };
 
 Layout layout(int32_t m, int32_t n, int64_t nnz) {
@@ -45,6 +46,8 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   for (int i = 0; i < 4; i++) L.q[i] = take(sizeof(int) * mx);
   L.ctacnt = take(sizeof(int) * MAX_CTAS);
   L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
+  L.hist_len = (int)std::min<long long>((long long)m + n + 2, 1 << 20);
+  L.hist = take(sizeof(int) * (size_t)L.hist_len);
   L.dbg = take(sizeof(int) * ((size_t)n + 1) + (getenv("MCM_TRACE") ? (size_t)atoi(getenv("MCM_TRACE")) * 24 : 0));
   L.total = o;
   return L;
@@ -190,7 +193,9 @@ void mcm_default_options(mcm_options_t *o) {
   o->gap = 0;
   o->final_check = 1;
   o->dead_skip = 1;
-  o->tail_max = 2048;
+  o->tail_max = 4096;
+  o->tail_ctas = 8;
+  o->compact_adapt = 1;
   o->compact_every = 0;
   o->grid_ctas = 0;
   o->max_loops = 0;
@@ -224,6 +229,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->gr_strategy != MCM_GR_ADAPTIVE && o->gr_strategy != MCM_GR_FIXED) return MCM_EINVAL;
   if (o->init < 0 || o->init > 2) return MCM_EINVAL;
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->max_loops < 0) return MCM_EINVAL;
+  if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -288,6 +294,7 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
     k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, cursor, cadj);
     CK(cudaGetLastError());
   }
+  CK(cudaMemsetAsync(ws + L.hist, 0, sizeof(int) * (size_t)L.hist_len, st));  // zero between gap uses
   CK(cudaStreamSynchronize(st));
   h->ms_setup = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
   memset(&h->stats, 0, sizeof(h->stats));
@@ -314,6 +321,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.ctacnt = (int *)(ws + L.ctacnt);
   p.ctrl = (Ctrl *)(ws + L.ctrl);
   p.dbgbuf = (int *)(ws + L.dbg);
+  p.hist = (int *)(ws + L.hist);
+  p.hist_len = L.hist_len;
   p.debug = getenv("MCM_DEBUG") ? atoi(getenv("MCM_DEBUG")) : 0;
   // MCM_TRACE=<n>: record up to n phase boundaries into the (otherwise idle during
   // a solve) debug buffer; dumped to MCM_TRACE_FILE after the solve (analysis only)
@@ -328,13 +337,40 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.k = o.k; p.gr_fixed = o.gr_strategy == MCM_GR_FIXED; p.shrink_min = o.shrink_min; p.init = o.init;
   p.gap = o.gap; p.final_check = o.final_check; p.dead_skip = o.dead_skip; p.tail_max = o.tail_max;
   p.compact_every = o.compact_every;
+  p.compact_adapt = o.compact_adapt;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
-  int grid = o.grid_ctas > 0 ? std::min(o.grid_ctas, h->max_grid) : h->max_grid;
+  int C = o.tail_ctas;
+  if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
+  int maxg = h->max_grid;
+  if (C > 1) {
+    // co-resident clusters of C CTAs (the tail group is cluster 0)
+    if (C > 8) CK(cudaFuncSetAttribute(gpr_kernel, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    cudaLaunchConfig_t q = {};
+    cudaLaunchAttribute qa[1];
+    qa[0].id = cudaLaunchAttributeClusterDimension;
+    qa[0].val.clusterDim.x = C; qa[0].val.clusterDim.y = 1; qa[0].val.clusterDim.z = 1;
+    q.gridDim = dim3(C); q.blockDim = dim3(NT); q.attrs = qa; q.numAttrs = 1;
+    int ncl = 0;
+    CK(cudaOccupancyMaxActiveClusters(&ncl, gpr_kernel, &q));
+    if (ncl < 1) return MCM_EINTERNAL;
+    maxg = std::min(maxg, ncl * C);
+  }
+  int grid = o.grid_ctas > 0 ? std::min(o.grid_ctas, maxg) : maxg;
+  grid = (grid / C) * C;
+  if (grid < C) return MCM_EINVAL;
+  p.tail_ctas = C;
   h->grid = grid;
   CK(cudaMemsetAsync(p.ctrl, 0, sizeof(Ctrl), st));
-  void *args[] = {&p};
-  CK(cudaLaunchCooperativeKernel((void *)gpr_kernel, grid, NT, args, 0, st));
+  cudaLaunchConfig_t cfg = {};
+  cudaLaunchAttribute at[2];
+  at[0].id = cudaLaunchAttributeCooperative;
+  at[0].val.cooperative = 1;
+  at[1].id = cudaLaunchAttributeClusterDimension;
+  at[1].val.clusterDim.x = C; at[1].val.clusterDim.y = 1; at[1].val.clusterDim.z = 1;
+  cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = 0; cfg.stream = st;
+  cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
+  CK(cudaLaunchKernelEx(&cfg, gpr_kernel, p));
   CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));
   CK(cudaStreamSynchronize(st));
   const Ctrl &c = h->host_ctrl;
@@ -360,7 +396,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     if (f) { fwrite(buf.data(), sizeof(long long), buf.size(), f); fclose(f); }
   }
   if (c.err) return c.err;
-  if (mode == MODE_RELABEL) return x[ST_MAXLEVEL];
+  if (mode == MODE_RELABEL || mode == MODE_GAP) return x[ST_MAXLEVEL];
   return x[ST_CARD];
 }
 
@@ -377,6 +413,12 @@ int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *r
   int64_t r = launch(h, (cudaStream_t)stream, MODE_RELABEL, rmatch, cmatch, psi_row, psi_col);
   if (r >= 0 && reached_free) *reached_free = h->host_ctrl.stat[ST_REACHED_FREE];
   return r;
+}
+
+int64_t mcm_gap_relabel(mcm_handle_t h, mcm_stream_t stream, int32_t *psi_row, int32_t *psi_col) {
+  if (!h) return MCM_EINVAL;
+  if ((h->m > 0 && !psi_row) || (h->n > 0 && !psi_col)) return MCM_EINVAL;
+  return launch(h, (cudaStream_t)stream, MODE_GAP, psi_row, psi_col, psi_row, psi_col);
 }
 
 int mcm_set_options(mcm_handle_t h, const mcm_options_t *o) {

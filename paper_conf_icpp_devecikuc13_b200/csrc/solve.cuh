@@ -26,7 +26,7 @@ constexpr int SMALL_DEG = 32;    // greedy: adjacency lists up to this length: o
 constexpr int BIG_DEG = 64;      // GR / push: longer lists go to the whole warp
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
 
-enum { MODE_SOLVE = 0, MODE_RELABEL = 1 };
+enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
 
 // statistics slots (Ctrl::stat)
 enum {
@@ -42,12 +42,13 @@ struct Ctrl {
   long long stat[ST_NSTAT];
   int err;                 // 0 or an MCM_* code
   u32 gcnt;                // exactness-guard list cursor (monotonic within a solve)
-  int pad[14];
+  int gmax, gmin;          // gap relabel: largest finite label, smallest empty label
+  int pad[12];
   long long dbg[8];        // debug checks: [0] count, [1] where, [2] loop, [3] vertex, [4] value
   // tail-mode handoff (CTA 0 -> grid)
   int ho_reason, ho_ph, ho_len, ho_ulen, ho_shrink, ho_ac0, ho_u0, ho_gl, ho_gd, ho_gn, ho_gc;
   u32 ho_base;
-  long long ho_loop, ho_iter;
+  long long ho_loop, ho_iter, ho_gapat;
 };
 
 struct Params {
@@ -57,13 +58,16 @@ struct Params {
   int *iA, *wl0, *wl1, *qa, *qb, *qc, *qd;
   int *ctacnt;
   int *dbgbuf;             // n ints (debug checks only)
+  int tail_ctas;           // CTAs of the tail group (= cluster 0 when > 1)
+  int *hist;               // gap relabel histogram (hist_len counters, zero between uses)
+  int hist_len;
   int debug;
   long long *trace;        // optional phase trace: {tag, size, t_end_ns} triples (MCM_TRACE)
   int trace_cap;
   Ctrl *ctrl;
   // options
   double k;
-  int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every;
+  int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt;
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -89,10 +93,11 @@ struct Solver {
   const int m, n, INF;
   // per-thread statistics (reduced at the end)
   long long s_push = 0, s_block = 0, s_dead = 0, s_scan = 0, s_slots = 0, s_free = 0;
-  long long s_grrows = 0, s_gredges = 0, s_grcols = 0, s_gyedges = 0;
+  long long s_grrows = 0, s_gredges = 0, s_grcols = 0, s_gyedges = 0, s_gapkill = 0;
   int ph = 0;  // phase counter: identical in every thread
   long long nbar = 0;
   int ttag = 0, tsz = 0, tn = 0;  // phase trace (lead thread only)
+  long long gaps_total = 0;
   __device__ __forceinline__ void trace(int tag, int sz) {
     ttag = tag; tsz = sz;
   }
@@ -112,23 +117,26 @@ struct Solver {
     if (GRID) {
       grid_sync(&p.ctrl->bar, false);
       nbar++;
+    } else if (p.tail_ctas > 1) {
+      // tail group = thread-block cluster 0: hardware cluster barrier (release /
+      // acquire at cluster scope covers the global writes of the cluster's CTAs)
+      asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
     } else {
       __syncthreads();
     }
     ph++;
-    if (GRID ? (blockIdx.x == 0 && threadIdx.x == 0) : (threadIdx.x == 0)) {
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
       u32 *r = p.ctrl->ring[(ph + 2) & 3];
       r[0] = r[1] = r[2] = r[3] = 0;
     }
-    if (!GRID) __syncthreads();
   }
   __device__ __forceinline__ u32 *ring_now(int j) { return &p.ctrl->ring[ph & 3][j]; }
   __device__ __forceinline__ u32 ring_prev(int j) { return ld_rlx(&p.ctrl->ring[(ph - 1) & 3][j]); }
 
   template <bool GRID>
-  __device__ __forceinline__ int cta() const { return GRID ? blockIdx.x : 0; }
+  __device__ __forceinline__ int cta() const { return blockIdx.x; }  // tail group = blocks [0, tail_ctas)
   template <bool GRID>
-  __device__ __forceinline__ int ncta() const { return GRID ? gridDim.x : 1; }
+  __device__ __forceinline__ int ncta() const { return GRID ? gridDim.x : p.tail_ctas; }
 
   // CTA total -> ring counter j (one atomic per CTA)
   __device__ __forceinline__ void add_count(long long x, int j) {
@@ -177,17 +185,21 @@ struct Solver {
       int val = (i < hi) ? f(i) : -1;
       int tot;
       int r = cta_rank<NT>(val != -1, sm.w, &tot);
-      if (val != -1) (GRID ? T[lo + run + r] : out[run + r]) = val;
+      if (val != -1) (C > 1 ? T[lo + run + r] : out[run + r]) = val;
       run += tot;
     }
-    if (GRID && threadIdx.x == 0) p.ctacnt[c] = run;
+    if (C > 1 && threadIdx.x == 0) p.ctacnt[c] = run;
     return run;
   }
   // Pass 2 (after a barrier): move T[lo_c ..] to out[offset_c ..]; returns the total.
   template <bool GRID>
   __device__ int compact_pass2(int len, const int *T, int *out, int run1, int *out2 = nullptr) {
-    if (!GRID) return run1;
-    const int C = gridDim.x, c = blockIdx.x;
+    const int C = ncta<GRID>(), c = cta<GRID>();
+    if (C == 1) {
+      if (out2)
+        for (int j = threadIdx.x; j < run1; j += NT) out2[j] = __ldcg(out + j);
+      return run1;
+    }
     const int chunk = (len + C - 1) / C;
     const int lo = min(len, c * chunk);
     long long before = 0, total = 0;
@@ -212,6 +224,17 @@ struct Solver {
   // else empty).  Labels start stale (psi = 0 < base).
   __device__ void init_state() {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    if (p.mode == MODE_GAP) {
+      for (int u = g; u < m; u += G) {
+        int l = p.rmatch_in[u];
+        st_rlx(p.rowst + u, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
+      }
+      for (int v = g; v < n; v += G) {
+        int l = p.cmatch_in[v];
+        st_rlx(p.colst + v, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
+      }
+      return;
+    }
     const bool given = (p.mode == MODE_RELABEL) || (p.init == 1);
     for (int u = g; u < m; u += G) st_rlx(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
     for (int v = g; v < n; v += G) {
@@ -630,9 +653,75 @@ struct Solver {
     barrier<true>();
   }
 
+  // ---------------------------------------------------------------- gap relabel
+  // Reading R14 of P:95-96 (the paper names GPU gap relabelling but gives no
+  // algorithm): count the vertices of every finite label l < H (rows carry even
+  // labels, columns odd); if some label g < L_max (the largest finite label) has
+  // no vertex, every label in (g, m+n) becomes m+n.  Valid because along any
+  // residual path labels drop by at most one per step (neighbourhood invariant,
+  // P:203-209, and psi(u) = psi(mu(u)) + 1 for matched rows), so a vertex above
+  // the gap cannot reach an unmatched row (label 0).  g = 0 (no unmatched row
+  // left) kills every active column.  Counting every vertex (dead columns
+  // included) can only hide gaps, never invent one.  Grid phases; returns g or -1.
+  __device__ int gap_relabel(u32 base) {
+    const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    const int H = p.hist_len;
+    Ctrl *c = p.ctrl;
+    if (blockIdx.x == 0 && threadIdx.x == 0) c->gmin = 0x7fffffff;
+    // per-CTA shared histogram of the low labels (the frontier staging buffer is
+    // idle here), flushed with one global atomic per non-empty bin
+    const int SH = min(QCAP, H);
+    for (int l = threadIdx.x; l < SH; l += NT) sm.q[l] = 0;
+    __syncthreads();
+    int lmax = -1;
+    for (int x = g; x < m + n; x += G) {
+      u64 w = ld_rlx(x < m ? p.rowst + x : p.colst + (x - m));
+      int l = lab(psi_of(w), base, INF);
+      if (l < INF) {
+        if (l < SH) atomicAdd(&sm.q[l], 1);
+        else if (l < H) atomicAdd(p.hist + l, 1);
+        lmax = max(lmax, l);
+      }
+    }
+    __syncthreads();
+    for (int l = threadIdx.x; l < SH; l += NT)
+      if (sm.q[l]) atomicAdd(p.hist + l, sm.q[l]);
+    __syncthreads();
+    if (threadIdx.x == 0) sm.qcnt = 0;
+    for (int o = 16; o > 0; o >>= 1) lmax = max(lmax, __shfl_xor_sync(0xffffffffu, lmax, o));
+    if (lane_id() == 0 && lmax >= 0) atomicMax(&c->gmax, lmax);
+    barrier<true>();
+    const int L = min((int)ld_rlx((const u32 *)&c->gmax), H);
+    int first = 0x7fffffff;
+    for (int l = g; l < L; l += G)
+      if (__ldcg(p.hist + l) == 0) { first = l; break; }
+    for (int o = 16; o > 0; o >>= 1) first = min(first, __shfl_xor_sync(0xffffffffu, first, o));
+    if (lane_id() == 0 && first != 0x7fffffff) atomicMin(&c->gmin, first);
+    barrier<true>();
+    const int gap = (int)ld_rlx((const u32 *)&c->gmin);
+    if (blockIdx.x == 0 && threadIdx.x == 0) c->gmax = 0;
+    long long killed = 0;
+    if (gap != 0x7fffffff) {
+      for (int x = g; x < m + n; x += G) {
+        u64 *a = x < m ? p.rowst + x : p.colst + (x - m);
+        u64 w = ld_rlx(a);
+        int l = lab(psi_of(w), base, INF);
+        if (l > gap && l < INF) { st_rlx(a, pack(mu_of(w), 0)); killed++; }  // psi 0 < base: infinite
+      }
+    }
+    for (int l = g; l < L; l += G) p.hist[l] = 0;
+    s_gapkill += killed;
+    barrier<true>();
+    return gap == 0x7fffffff ? -1 : gap;
+  }
+
   // ---------------------------------------------------------------- tail mode
-  enum { R_NONE = 0, R_TERM = 1, R_NEEDGR = 2, R_ESC = 3, R_CAP = 4 };
-  __device__ __forceinline__ int tail_f() const { return p.tail_max * 4 > 4096 ? p.tail_max * 4 : 4096; }
+  enum { R_NONE = 0, R_TERM = 1, R_NEEDGR = 2, R_ESC = 3, R_CAP = 4, R_GAP = 5 };
+  // gap relabel schedule (R14): once, halfway between two GRs
+  __device__ __forceinline__ long long gap_at(long long loop, long long iterGR) const {
+    return (p.gap && iterGR - loop >= 2) ? loop + (iterGR - loop) / 2 : -1;
+  }
+  __device__ __forceinline__ int tail_f() const { return p.tail_max * 2; }
 
   // All CTAs call.  CTA 0 runs Alg. 7 iterations alone -- fix with compaction at
   // every step, push, and GRs whose frontiers stay narrow -- with __syncthreads
@@ -641,17 +730,19 @@ struct Solver {
   // grew past tail_f(): R_ESC hands the BFS state over), when no active column is
   // left (R_TERM) or at the iteration cap (R_CAP).  CTA 0 then publishes its
   // control registers and every CTA adopts them after the barrier.
-  __device__ int tail_episode(long long &loop, long long &iterGR, int &len, int &ulen, u32 &base, bool &shrink,
+  __device__ int tail_episode(long long &loop, long long &iterGR, long long &gapAt, int &len, int &ulen, u32 &base,
+                              bool &shrink,
                               int *&Ac, int *&Ap, int *&U, int *&T, int *Qa, int *Qb, GRState &gst, long long &grs,
                               long long &levels, long long &shrinks, long long &tail_loops, long long &ns_gr,
                               long long &ns_loop) {
     const u32 stride = (u32)(m + n + 2);
     int reason = R_NONE;
     Ctrl *c = p.ctrl;
-    if (blockIdx.x == 0) {
+    if (blockIdx.x < p.tail_ctas) {
       const int limit = tail_f();
       for (;;) {
         if (loop >= p.max_loops) { reason = R_CAP; break; }
+        if (loop == gapAt) { reason = R_GAP; break; }
         if (loop == iterGR) {
           if (ulen > limit || (u64)base + 2ull * stride >= 0xfffffff0ull) { reason = R_NEEDGR; break; }
           u64 g0 = gtime();
@@ -662,6 +753,7 @@ struct Solver {
           int ml = gst.deepest + 2;
           grs++; levels += ml / 2;
           iterGR = loop + iter_gap(ml);
+          gapAt = gap_at(loop, iterGR);
           shrink = true;
           base += stride;
         }
@@ -669,9 +761,14 @@ struct Solver {
         const int lp = (int)loop;
         if (threadIdx.x == 0) s_slots += len;
         trace(3, len);
-        int r1 = compact_pass1<false>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, nullptr, Ac);
+        int r1 = compact_pass1<false>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
         barrier<false>();
-        len = r1;
+        if (p.tail_ctas > 1) {
+          len = compact_pass2<false>(len, T, Ac, r1);
+          barrier<false>();
+        } else {
+          len = r1;
+        }
         if (shrink) { shrinks++; shrink = false; }
         if (len == 0) { reason = R_TERM; ns_loop += (long long)(gtime() - l0); break; }
         trace(4, len);
@@ -685,7 +782,7 @@ struct Solver {
       if (threadIdx.x == 0) {
         c->ho_reason = reason; c->ho_ph = ph; c->ho_len = len; c->ho_ulen = ulen; c->ho_shrink = shrink;
         c->ho_ac0 = (Ac == p.wl0); c->ho_u0 = (U == p.qa); c->ho_loop = loop; c->ho_iter = iterGR;
-        c->ho_base = base; c->ho_gl = gst.lvl; c->ho_gd = gst.deepest; c->ho_gn = gst.nlen; c->ho_gc = gst.cur_is_a;
+        c->ho_base = base; c->ho_gapat = gapAt; c->ho_gl = gst.lvl; c->ho_gd = gst.deepest; c->ho_gn = gst.nlen; c->ho_gc = gst.cur_is_a;
         for (int j = 0; j < 4; j++) c->ring[j][0] = c->ring[j][1] = c->ring[j][2] = c->ring[j][3] = 0;
       }
     }
@@ -705,6 +802,7 @@ struct Solver {
     U = u0 ? p.qa : p.qb; T = u0 ? p.qb : p.qa;
     loop = ld_rlx(&c->ho_loop);
     iterGR = ld_rlx(&c->ho_iter);
+    gapAt = ld_rlx(&c->ho_gapat);
     base = ld_rlx(&c->ho_base);
     gst.lvl = (int)ld_rlx((const u32 *)&c->ho_gl); gst.deepest = (int)ld_rlx((const u32 *)&c->ho_gd);
     gst.nlen = (int)ld_rlx((const u32 *)&c->ho_gn); gst.cur_is_a = (int)ld_rlx((const u32 *)&c->ho_gc);
@@ -737,6 +835,13 @@ struct Solver {
     u32 base = 1;  // epoch of the next GR
     const u32 stride = (u32)(m + n + 2);
 
+    if (p.mode == MODE_GAP) {  // mcm_gap_relabel: labels in, labels out
+      int gl = gap_relabel(1);
+      write_labels(1);
+      if (lead) p.ctrl->stat[ST_MAXLEVEL] = gl;
+      finish_stats(0, 0, 0, 0, 0, 0, 0, 0, 0, 0, 0);
+      return;
+    }
     if (p.mode == MODE_RELABEL) {
       int g;
       int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, nullptr, g);
@@ -753,8 +858,8 @@ struct Solver {
     u64 t1 = gtime();
     ns_init = (long long)(t1 - t0);
 
-    long long loop = 0, iterGR = 0, tail_loops = 0;
-    bool shrink = false;
+    long long loop = 0, iterGR = 0, tail_loops = 0, gapAt = -1, gaps = 0;
+    bool shrink = false, compact_next = false;
     GRState gst;
     int reason = R_NONE;
     for (;;) {
@@ -766,13 +871,20 @@ struct Solver {
       reason = R_NONE;
       // ---- tail episode: a short worklist runs on CTA 0 alone (CTA barriers)
       if (p.tail_max > 0 && len <= p.tail_max && !(loop == iterGR && ulen > tail_f())) {
-        reason = tail_episode(loop, iterGR, len, ulen, base, shrink, Ac, Ap, U, T, Qa, Qb, gst, grs, levels,
+        reason = tail_episode(loop, iterGR, gapAt, len, ulen, base, shrink, Ac, Ap, U, T, Qa, Qb, gst, grs, levels,
                               shrinks, tail_loops, ns_gr, ns_loop);
         if (reason == R_CAP) {
           if (lead) p.ctrl->err = -5;
           break;
         }
         if (reason == R_TERM) terminated = true;
+      }
+      if (!terminated && loop == gapAt) {                              // gap relabel (R14)
+        u64 g0 = gtime();
+        if (gap_relabel(base - stride) >= 0) gaps++;
+        gapAt = -1;
+        ns_gr += (long long)(gtime() - g0);
+        if (p.tail_max > 0 && len <= p.tail_max && loop != iterGR) continue;
       }
       if (!terminated) {
         if (reason == R_ESC || loop == iterGR) {                       // Alg. 7 l.6
@@ -788,6 +900,7 @@ struct Solver {
           }
           grs++; levels += ml / 2;
           iterGR = loop + iter_gap(ml);                                // l.8
+          gapAt = gap_at(loop, iterGR);
           shrink = true;                                               // l.9
           base += stride;
           ns_gr += (long long)(gtime() - g0);
@@ -796,7 +909,7 @@ struct Solver {
         const u32 cur = base - stride;  // epoch of the labels in use
         u64 l0 = gtime();
         int act;
-        if ((shrink && p.shrink_min >= 0 && len >= p.shrink_min) || p.compact_every) {  // l.11
+        if ((shrink && p.shrink_min >= 0 && len >= p.shrink_min) || p.compact_every || compact_next) {  // l.11
           const int lp = (int)loop;
           int r1 = compact_pass1<true>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
           s_slots += 0;
@@ -806,6 +919,7 @@ struct Solver {
           act = len;
           if (shrink) shrinks++;
           shrink = false;                                              // l.13
+          compact_next = false;
           // Ac was rewritten by CTAs other than the pushing one: order it before PUSH
           barrier<true>();
         } else {
@@ -813,6 +927,9 @@ struct Solver {
           fix_plain<true>(len, Ac, Ap, (int)loop, 0);                  // l.15
           barrier<true>();
           act = (int)ring_prev(0);
+          // adaptive compaction (beyond the paper's post-GR shrink): when most slots
+          // are empty, the next fix step compacts, so the tail group can take over
+          if (p.compact_adapt && act > 0 && (long long)act * 4 < len && len > p.tail_max) compact_next = true;
         }
         debug_check(3, loop, Ac, len);
         if (act != 0) {
@@ -851,9 +968,11 @@ struct Solver {
       if (lead) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
       len = gcount;
       iterGR = loop + iter_gap(ml);
+      gapAt = gap_at(loop, iterGR);
       shrink = false;
     }
     loops += tail_loops;
+    gaps_total = gaps;
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
     finish_stats(loops, grs, levels, shrinks, guard_re, init_card, ns_init, ns_gr, ns_loop, (long long)(gtime() - tA),
@@ -880,6 +999,7 @@ struct Solver {
     if (blockIdx.x == 0 && threadIdx.x == 0) {
       long long *st = p.ctrl->stat;
       st[ST_LOOPS] = loops; st[ST_GRS] = grs; st[ST_LEVELS] = levels; st[ST_SHRINKS] = shrinks;
+      st[ST_GAPS] = gaps_total;
       st[ST_GUARD] = guard_re; st[ST_INITCARD] = init_card; st[ST_NS_INIT] = ns_init; st[ST_NS_GR] = ns_gr;
       st[ST_NS_LOOP] = ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = tail_loops;
       st[ST_BARRIERS] = nbar;

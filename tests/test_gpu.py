@@ -105,7 +105,8 @@ def test_solve_default(name, mk):
 OPTION_SETS = [
     dict(k=0.3), dict(k=2.0), dict(gr_strategy="fixed", k=10), dict(gr_strategy="fixed", k=50), dict(shrink_min=-1),
     dict(shrink_min=1), dict(compact_every=1), dict(init="empty"), dict(final_check=0), dict(dead_skip=0),
-    dict(tail_max=0), dict(tail_max=100000), dict(grid_ctas=1), dict(grid_ctas=7), dict(gap=1),
+    dict(tail_max=0), dict(tail_max=100000), dict(grid_ctas=1), dict(grid_ctas=7), dict(gap=1), dict(tail_ctas=1),
+    dict(tail_ctas=2), dict(tail_ctas=16), dict(compact_adapt=0), dict(grid_ctas=16, tail_ctas=16),
 ]
 
 
@@ -210,3 +211,41 @@ def test_full_size_config(name):
     if mm is None:
         mm = oracle.hopcroft_karp(g)[0]
     check_solve(g, mm)
+
+
+# ---------------------------------------------------------------- gap relabel, bit-exact
+def test_gap_relabel_bit_exact():
+    """mcm_gap_relabel (the routine the solve runs with gap=1) against the oracle's
+    reading R14 on label arrays with and without holes."""
+    rng = np.random.default_rng(77)
+    for t in range(12):
+        g = synth.config("C1", 0.05) if t % 2 else synth.random_small(300, 200, 0.02, t)
+        ip, ix = dev(g)
+        mt = pkg.Matcher(ip, ix, g.m, g.n)
+        INF = g.m + g.n
+        top = int(rng.integers(2, 60))
+        pr = rng.integers(0, top, g.m).astype(np.int32)
+        pc = rng.integers(0, top, g.n).astype(np.int32)
+        hole = int(rng.integers(0, top))
+        if t % 3 != 2:  # punch a hole (t % 3 == 2: maybe none)
+            pr[pr == hole] = hole + 1
+            pc[pc == hole] = hole + 1
+        pr[rng.random(g.m) < 0.1] = INF + 3
+        pc[rng.random(g.n) < 0.1] = -1
+        gl, dpr, dpc = mt.gap_relabel(torch.from_numpy(pr), torch.from_numpy(pc))
+        egl, epr, epc = oracle.gap_relabel(g.m, g.n, pr, pc)
+        assert gl == egl, (t, gl, egl)
+        assert np.array_equal(dpr.cpu().numpy(), epr) and np.array_equal(dpc.cpu().numpy(), epc), t
+        mt.close()
+
+
+def test_gap_solves_exact_without_guard():
+    """Soundness on the GPU: with gap relabelling on and the exactness guard off the
+    cardinality is still the maximum (an unsound gap would kill augmentable columns)."""
+    graphs = [synth.config("C1"), synth.config("C4", 1 / 128), synth.hall_violator(5000, 300, 77, 1),
+              synth.from_pairs(3000, 5000, np.arange(9000) % 3000, (np.arange(9000) * 7) % 5000),
+              synth.config("C3", 0.002)]
+    for g in graphs:
+        card, st = check_solve(g, gap=1, final_check=0)
+        card2, st2 = check_solve(g, gap=1, final_check=1)
+        assert st2["guard_reactivated"] == 0

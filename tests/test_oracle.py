@@ -278,3 +278,47 @@ def test_full_size_oracles_agree(name):
     if g.mm is not None:
         assert c1 == g.mm
     assert oracle.konig_cover(g, rm, cm)[0] == c1
+
+
+# ---------------------------------------------------------------- gap relabel (reading R14)
+def test_gap_hand_examples():
+    """Worked by hand from reading R14: INF = m+n."""
+    g, pr, pc = oracle.gap_relabel(3, 2, [0, 2, 4], [1, 3])  # INF 5, labels 0..4 all present
+    assert g == -1 and list(pr) == [0, 2, 4] and list(pc) == [1, 3]
+    g, pr, pc = oracle.gap_relabel(3, 2, [0, 4, 9], [1, 3])  # label 2 empty, L_max 4
+    assert g == 2 and list(pr) == [0, 5, 5] and list(pc) == [1, 5]
+    g, pr, pc = oracle.gap_relabel(2, 2, [2, 4], [1, 3])  # no label 0: no unmatched row left
+    assert g == 0 and list(pr) == [4, 4] and list(pc) == [4, 4]
+    g, pr, pc = oracle.gap_relabel(2, 2, [0, -1], [1, 7])  # negatives / >= INF are infinite
+    assert g == -1 and list(pr) == [0, 4] and list(pc) == [1, 4]
+
+
+def test_gap_is_noop_on_exact_labels():
+    """BFS layers are contiguous, so exact GR labels never contain a gap."""
+    rng = np.random.default_rng(31)
+    for t in range(100):
+        m, n = int(rng.integers(1, 40)), int(rng.integers(1, 40))
+        g = synth.random_small(m, n, float(rng.uniform(0.03, 0.3)), int(rng.integers(1 << 30)))
+        rm, cm = _random_mu(g, rng)
+        pr, pc, _, _ = oracle.global_relabel(g, rm, cm)
+        gl, pr2, pc2 = oracle.gap_relabel(g.m, g.n, pr, pc)
+        assert gl == -1 and np.array_equal(pr, pr2) and np.array_equal(pc, pc2)
+
+
+def test_gpr_serial_with_gap_stays_exact():
+    """Soundness pin: G-PR with gap relabelling (R14) still reaches the maximum
+    cardinality (HK) -- an unsound gap would kill an augmentable column."""
+    rng = np.random.default_rng(41)
+    total_gaps = 0
+    graphs = [synth.config("C4", 1 / 2048), synth.config("C1", 0.3), synth.hall_violator(900, 60, 21, 4)]
+    for _ in range(60):
+        m, n = int(rng.integers(2, 60)), int(rng.integers(2, 60))
+        graphs.append(synth.random_small(m, n, float(rng.uniform(0.02, 0.2)), int(rng.integers(1 << 30))))
+    for g in graphs:
+        mm = oracle.hopcroft_karp(g)[0]
+        for k in (0.7, 3.0, 10.0):
+            c, rm, cm, st = oracle.gpr_serial(g, k=k, gap=True)
+            assert c == mm, (g.name, k, c, mm, st)
+            assert oracle.check_matching(g, rm, cm) == mm
+            total_gaps += st["gaps"]
+    assert total_gaps > 0  # the gap path was exercised
