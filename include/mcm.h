@@ -89,8 +89,9 @@ typedef struct {
   int32_t compact_every;/* 1: compact the worklist at every fix step (an option beyond
                            the paper's post-GR shrink); default 0 */
   int32_t grid_ctas;    /* CTAs of the persistent kernel; 0 (default) = all co-resident */
-  int32_t tail_ctas;    /* CTAs of the tail group: 1 = one CTA (__syncthreads), 2..16 = a
-                           thread-block cluster (hardware cluster barrier); default 8 */
+  int32_t tail_ctas;    /* CTAs of the tail group: 1 (default) = one CTA (__syncthreads);
+                           2..16 (power of 2) = a thread-block cluster with the hardware
+                           cluster barrier (the grid then shrinks to whole clusters) */
   int32_t compact_adapt;/* 1 (default): compact the worklist at the next fix step when
                            fewer than 1/4 of its slots hold an active column */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
@@ -176,6 +177,10 @@ int mcm_get_stats(mcm_handle_t h, mcm_stats_t *out);
 int mcm_destroy(mcm_handle_t h);
 
 const char *mcm_strerror(int code);
+
+/* sizeof(mcm_options_t) and sizeof(mcm_stats_t) as compiled into the library, so a
+ * binding can verify its struct mirrors (returns MCM_OK). */
+int mcm_abi_sizes(size_t *options_size, size_t *stats_size);
 
 #ifdef __cplusplus
 }

@@ -58,9 +58,7 @@ class Stats(ctypes.Structure):
         "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers", "gr_rows", "gr_edges",
         "gr_cols", "greedy_edges")] + [
         (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
-        ("grid_ctas", ctypes.c_int32),
-        ("tail_ctas", ctypes.c_int32),
-        ("compact_adapt", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
+        ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
 
     def as_dict(self):
         return {f: getattr(self, f) for f, _ in self._fields_}
@@ -106,6 +104,13 @@ def lib():
         L.mcm_destroy.restype = ctypes.c_int
         L.mcm_strerror.argtypes = [ctypes.c_int]
         L.mcm_strerror.restype = ctypes.c_char_p
+        L.mcm_abi_sizes.argtypes = [P(sz), P(sz)]
+        L.mcm_abi_sizes.restype = ctypes.c_int
+        so, ss = sz(0), sz(0)
+        L.mcm_abi_sizes(ctypes.byref(so), ctypes.byref(ss))
+        if so.value != ctypes.sizeof(Options) or ss.value != ctypes.sizeof(Stats):
+            raise ImportError(f"libmcm.so ABI mismatch: options {so.value} vs {ctypes.sizeof(Options)}, "
+                              f"stats {ss.value} vs {ctypes.sizeof(Stats)}")
         _lib = L
     return _lib
 

@@ -194,7 +194,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->final_check = 1;
   o->dead_skip = 1;
   o->tail_max = 4096;
-  o->tail_ctas = 8;
+  o->tail_ctas = 1;
   o->compact_adapt = 1;
   o->compact_every = 0;
   o->grid_ctas = 0;
@@ -436,6 +436,12 @@ int mcm_set_k(mcm_handle_t h, double k) {
 int mcm_get_stats(mcm_handle_t h, mcm_stats_t *out) {
   if (!h || !out) return MCM_EINVAL;
   *out = h->stats;
+  return MCM_OK;
+}
+
+int mcm_abi_sizes(size_t *options_size, size_t *stats_size) {
+  if (options_size) *options_size = sizeof(mcm_options_t);
+  if (stats_size) *stats_size = sizeof(mcm_stats_t);
   return MCM_OK;
 }
 

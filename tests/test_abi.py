@@ -19,7 +19,8 @@ def declared_functions():
 
 def test_header_declares_the_boundary():
     names = declared_functions()
-    for f in ["mcm_create", "mcm_solve", "mcm_set_k", "mcm_get_stats", "mcm_destroy", "mcm_strerror",
+    for f in ["mcm_create", "mcm_solve", "mcm_set_k", "mcm_get_stats", "mcm_destroy", "mcm_strerror", "mcm_abi_sizes",
+              "mcm_gap_relabel",
               "mcm_default_options", "mcm_workspace_bytes", "mcm_global_relabel", "mcm_set_options"]:
         assert f in names
 
