@@ -144,6 +144,22 @@ def setup_bytes(m, n, nnz):
     return int(4 * (m + 1) * 4 + 4 * nnz * 8 + 12 * n)
 
 
+def reduce_over_ranks(t_step, t_e2e, t_solve, t_create, nnz, world, device):
+    """Max over ranks of every time (the job is as slow as its slowest rank), sum of
+    the units (edges) all ranks processed.  No data-path collective: this runs once,
+    after the timed region."""
+    import torch
+
+    vals = torch.tensor([t_step, t_e2e, t_solve, t_create, nnz], dtype=torch.float64, device=device)
+    if world > 1:
+        mx = vals.clone()
+        torch.distributed.all_reduce(mx, op=torch.distributed.ReduceOp.MAX)
+        sm = vals.clone()
+        torch.distributed.all_reduce(sm, op=torch.distributed.ReduceOp.SUM)
+        return mx[0].item(), mx[1].item(), mx[2].item(), mx[3].item(), sm[4].item()
+    return t_step, t_e2e, t_solve, t_create, nnz
+
+
 def run_ours(args, rank, world, local_rank):
     import torch
 
@@ -232,17 +248,9 @@ def run_ours(args, rank, world, local_rank):
             e2e_ms.append(a.elapsed_time(b))
     t_e2e = sum(e2e_ms) / len(e2e_ms)
 
-    # ---- max over ranks
-    vals = torch.tensor([t_step, t_e2e, float(g.nnz), t_solve, t_create], dtype=torch.float64, device=dev)
-    if world > 1:
-        mx = vals.clone()
-        torch.distributed.all_reduce(mx, op=torch.distributed.ReduceOp.MAX)
-        sm = vals.clone()
-        torch.distributed.all_reduce(sm, op=torch.distributed.ReduceOp.SUM)
-        t_step_max, t_e2e_max, t_solve_max, t_create_max = mx[0].item(), mx[1].item(), mx[3].item(), mx[4].item()
-        nnz_total = sm[2].item()
-    else:
-        t_step_max, t_e2e_max, t_solve_max, t_create_max, nnz_total = t_step, t_e2e, t_solve, t_create, float(g.nnz)
+    # ---- max over ranks (times), sum over ranks (units processed)
+    t_step_max, t_e2e_max, t_solve_max, t_create_max, nnz_total = reduce_over_ranks(
+        t_step, t_e2e, t_solve, t_create, float(g.nnz), world, dev)
     if rank != 0:
         return None
 
