@@ -42,6 +42,7 @@ class Options(ctypes.Structure):
         ("final_check", ctypes.c_int32),
         ("dead_skip", ctypes.c_int32),
         ("tail_max", ctypes.c_int32),
+        ("tail_f", ctypes.c_int32),
         ("compact_every", ctypes.c_int32),
         ("grid_ctas", ctypes.c_int32),
         ("tail_ctas", ctypes.c_int32),

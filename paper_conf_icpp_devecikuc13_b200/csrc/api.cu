@@ -43,7 +43,7 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   L.iA = take(sizeof(int) * (size_t)n);
   L.wl0 = take(sizeof(int) * (size_t)n);
   L.wl1 = take(sizeof(int) * (size_t)n);
-  for (int i = 0; i < 4; i++) L.q[i] = take(sizeof(int) * mx);
+  for (int i = 0; i < 4; i++) L.q[i] = take((i < 2 ? sizeof(int) : sizeof(int4)) * mx);  // q2, q3: int4 frontiers
   L.ctacnt = take(sizeof(int) * MAX_CTAS);
   L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
   L.hist_len = (int)std::min<long long>((long long)m + n + 2, 1 << 20);
@@ -193,7 +193,8 @@ void mcm_default_options(mcm_options_t *o) {
   o->gap = 0;
   o->final_check = 1;
   o->dead_skip = 1;
-  o->tail_max = 4096;
+  o->tail_max = 512;
+  o->tail_f = 0;
   o->tail_ctas = 1;
   o->compact_adapt = 1;
   o->compact_every = 0;
@@ -228,7 +229,8 @@ static int check_opts(const mcm_options_t *o) {
   if (!(o->k > 0) || !std::isfinite(o->k)) return MCM_EINVAL;
   if (o->gr_strategy != MCM_GR_ADAPTIVE && o->gr_strategy != MCM_GR_FIXED) return MCM_EINVAL;
   if (o->init < 0 || o->init > 2) return MCM_EINVAL;
-  if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->max_loops < 0) return MCM_EINVAL;
+  if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
+    return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
   return MCM_OK;
 }
@@ -251,7 +253,8 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   CK(cudaGetDevice(&h->dev));
   CK(cudaDeviceGetAttribute(&h->sms, cudaDevAttrMultiProcessorCount, h->dev));
   int per_sm = 0;
-  CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel, NT, 0));
+  CK(cudaFuncSetAttribute(gpr_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Smem)));
+  CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel, NT, sizeof(Smem)));
   if (per_sm < 1) return MCM_EINTERNAL;
   h->max_grid = h->sms * (per_sm > 2 ? 2 : per_sm);  // one or two CTAs per SM (MCM_MINB)
   if (h->max_grid > MAX_CTAS) h->max_grid = MAX_CTAS;
@@ -338,6 +341,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.gap = o.gap; p.final_check = o.final_check; p.dead_skip = o.dead_skip; p.tail_max = o.tail_max;
   p.compact_every = o.compact_every;
   p.compact_adapt = o.compact_adapt;
+  p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
   int C = o.tail_ctas;
@@ -351,6 +355,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     qa[0].id = cudaLaunchAttributeClusterDimension;
     qa[0].val.clusterDim.x = C; qa[0].val.clusterDim.y = 1; qa[0].val.clusterDim.z = 1;
     q.gridDim = dim3(C); q.blockDim = dim3(NT); q.attrs = qa; q.numAttrs = 1;
+    q.dynamicSmemBytes = sizeof(Smem);
     int ncl = 0;
     CK(cudaOccupancyMaxActiveClusters(&ncl, gpr_kernel, &q));
     if (ncl < 1) return MCM_EINTERNAL;
@@ -368,7 +373,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   at[0].val.cooperative = 1;
   at[1].id = cudaLaunchAttributeClusterDimension;
   at[1].val.clusterDim.x = C; at[1].val.clusterDim.y = 1; at[1].val.clusterDim.z = 1;
-  cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = 0; cfg.stream = st;
+  cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = sizeof(Smem); cfg.stream = st;
   cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
   CK(cudaLaunchKernelEx(&cfg, gpr_kernel, p));
   CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));

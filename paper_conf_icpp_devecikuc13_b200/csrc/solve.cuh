@@ -21,7 +21,8 @@ namespace mcm {
 
 constexpr int NT = 512;          // threads per CTA
 constexpr int NWARP = NT / 32;
-constexpr int QCAP = 4096;       // shared staging for the next BFS frontier
+constexpr int QCAP = 16384;      // shared staging (ints, 64 KB, dynamic smem): next BFS frontier, gap histogram
+constexpr int QCAP4 = QCAP / 4;  // ... as int4 frontier entries
 constexpr int SMALL_DEG = 32;    // greedy: adjacency lists up to this length: one thread
 constexpr int BIG_DEG = 64;      // GR / push: longer lists go to the whole warp
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
@@ -45,20 +46,20 @@ struct Ctrl {
   int gmax, gmin;          // gap relabel: largest finite label, smallest empty label
   int pad[12];
   long long dbg[8];        // debug checks: [0] count, [1] where, [2] loop, [3] vertex, [4] value
-  // tail-mode handoff (CTA 0 -> grid)
-  int ho_reason, ho_ph, ho_len, ho_ulen, ho_shrink, ho_ac0, ho_u0, ho_gl, ho_gd, ho_gn, ho_gc;
-  u32 ho_base;
-  long long ho_loop, ho_iter, ho_gapat;
+  // tail-mode handoff (tail group -> grid): reason, phase counter, Ctl image
+  int ho_reason, ho_ph;
+  long long ho[32];
 };
 
 struct Params {
   int m, n, mode;
   const int *rptr, *radj, *cptr, *cadj;
   u64 *rowst, *colst;
-  int *iA, *wl0, *wl1, *qa, *qb, *qc, *qd;
+  int *iA, *wl0, *wl1, *qa, *qb, *qc, *qd;  // qc, qd: int4 BFS frontiers
   int *ctacnt;
   int *dbgbuf;             // n ints (debug checks only)
   int tail_ctas;           // CTAs of the tail group (= cluster 0 when > 1)
+  int tail_f;              // GR frontier limit of the tail group (0: 2 * tail_max)
   int *hist;               // gap relabel histogram (hist_len counters, zero between uses)
   int hist_len;
   int debug;
@@ -77,7 +78,7 @@ struct Params {
 struct Smem {
   long long red[NWARP];
   int w[NWARP];
-  int q[QCAP];
+  alignas(16) int q[QCAP];
   int qcnt, qbase, tmp;
 };
 
@@ -153,17 +154,32 @@ struct Solver {
   }
 
   // ---------------------------------------------------------------- staging
-  __device__ __forceinline__ void stage(int x, int *next, u32 *gcnt) {
-    int q = atomicAdd(&sm.qcnt, 1);
-    if (q < QCAP) sm.q[q] = x;
-    else next[atomicAdd(gcnt, 1u)] = x;  // overflow: direct append
+  // BFS frontier entries are {row, rptr[row], rptr[row+1], 0}: the producer loads
+  // the adjacency bounds of a row it discovers in parallel with its mate check, so
+  // the next level starts one dependent load earlier.
+  __device__ __forceinline__ void stage(int4 x, int4 *next, u32 *gcnt) {
+    // warp-aggregated: one shared atomic per group of converged lanes
+    cg::coalesced_group g = cg::coalesced_threads();
+    int base = 0;
+    if (g.thread_rank() == 0) base = atomicAdd(&sm.qcnt, (int)g.size());
+    base = g.shfl(base, 0);
+    int q = base + (int)g.thread_rank();
+    if (q < QCAP4) {
+      reinterpret_cast<int4 *>(sm.q)[q] = x;
+    } else {  // overflow: direct append, again one global atomic per group
+      cg::coalesced_group o = cg::coalesced_threads();
+      u32 gb = 0;
+      if (o.thread_rank() == 0) gb = atomicAdd(gcnt, (u32)o.size());
+      gb = o.shfl(gb, 0);
+      next[gb + o.thread_rank()] = x;
+    }
   }
-  __device__ __forceinline__ void flush(int *next, u32 *gcnt) {
+  __device__ __forceinline__ void flush(int4 *next, u32 *gcnt) {
     __syncthreads();
-    int c = min(sm.qcnt, QCAP);
+    int c = min(sm.qcnt, QCAP4);
     if (threadIdx.x == 0) sm.qbase = c ? (int)atomicAdd(gcnt, (u32)c) : 0;
     __syncthreads();
-    for (int j = threadIdx.x; j < c; j += NT) next[sm.qbase + j] = sm.q[j];
+    for (int j = threadIdx.x; j < c; j += NT) next[sm.qbase + j] = reinterpret_cast<const int4 *>(sm.q)[j];
     __syncthreads();
     if (threadIdx.x == 0) sm.qcnt = 0;
     __syncthreads();
@@ -236,7 +252,9 @@ struct Solver {
       return;
     }
     const bool given = (p.mode == MODE_RELABEL) || (p.init == 1);
-    for (int u = g; u < m; u += G) st_rlx(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
+    for (int u = g; u < m; u += G) {
+      st_rlx(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
+    }
     for (int v = g; v < n; v += G) {
       st_rlx(p.colst + v, pack(given ? p.cmatch_in[v] : -1, 0));
       p.iA[v] = -1;  // R12
@@ -327,17 +345,21 @@ struct Solver {
     return G == 32 ? 0xffffffffu : (((1u << G) - 1u) << (lane_id() & ~(G - 1)));
   }
 
+  // One BFS level (Alg. 5).  lvl == 0: `cur0` is the unmatched-row list U (rows
+  // matched since are dropped, the others get label 0 and go to Uout); lvl > 0:
+  // `cur4` holds the frontier entries of the previous level.
   template <bool GRID>
-  __device__ void gr_level(const int *cur, int curlen, int lvl, u32 base, int *next, u32 *ncnt, int *Uout,
-                           u32 *ucnt, int *guard, u32 *gcnt) {
+  __device__ void gr_level(const int *cur0, const int4 *cur4, int curlen, int lvl, u32 base, int4 *next, u32 *ncnt,
+                           int *Uout, u32 *ucnt, int *guard, u32 *gcnt) {
     const int lane = lane_id();
     const u32 lc = base + lvl + 1, lr = base + lvl + 2;
     const int G = pick_group(curlen, ncta<GRID>() * NT);
     const int gl = lane & (G - 1), per_tile = NT / G;
     for (int t = cta<GRID>() * per_tile; t < curlen; t += ncta<GRID>() * per_tile) {
       int i = t + (int)threadIdx.x / G;
-      int u = (i < curlen) ? ld_cg(cur + i) : -1;
+      int u = -1, s = 0, e = 0;
       if (lvl == 0) {
+        u = (i < curlen) ? ld_cg(cur0 + i) : -1;
         bool keep = false;
         if (u >= 0) {
           if (mu_of(ld_rlx(p.rowst + u)) == -1) {
@@ -351,32 +373,35 @@ struct Solver {
         if (threadIdx.x == 0) sm.tmp = tot ? (int)atomicAdd(ucnt, (u32)tot) : 0;
         __syncthreads();
         if (keep) Uout[sm.tmp + r] = u;
+        if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
+      } else if (i < curlen) {
+        int4 q = __ldcg(cur4 + i);
+        u = q.x; s = q.y; e = q.z;
       }
-      int s = 0, e = 0;
-      if (u >= 0) {
-        s = ld_ro(p.rptr + u);
-        e = ld_ro(p.rptr + u + 1);
-        if (gl == 0) { s_grrows++; s_gredges += e - s; }
-      }
+      if (u >= 0 && gl == 0) { s_grrows++; s_gredges += e - s; }
       const bool big = u >= 0 && G < 32 && e - s > BIG_DEG;
-      if (u >= 0 && !big) expand(s + gl, e, G, lc, lr, next, ncnt, guard, gcnt);
+      if (u >= 0 && !big) expand(s + gl, e, G, lc, lr, next, ncnt, guard, gcnt, G >= 4);
       unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
       while (bigm) {  // long lists: the whole warp
         int bl = __ffs(bigm) - 1;
         bigm &= bigm - 1;
         int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
-        expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt);
+        expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt, false);
       }
       flush(next, ncnt);
     }
   }
-  // Visit radj[j], j = j0, j0+step, ... < e, KB at a time: the KB column loads, then
-  // the KB claims (CAS), then the KB mate checks are each issued back to back.
-  __device__ __forceinline__ void expand(int j0, int e, int step, u32 lc, u32 lr, int *next, u32 *ncnt, int *guard,
-                                         u32 *gcnt) {
+  // Visit radj[j], j = j0, j0+step, ... < e, KB at a time.  A CAS claims each
+  // column once per GR (so every row joins the next frontier once and every
+  // reached unmatched column is counted once); the mate check and the mate's
+  // adjacency bounds are loaded in the same round trip as the CAS (they depend only
+  // on the column word), so a level costs: column loads -> {CAS, mate, bounds}.
+  __device__ __forceinline__ void expand(int j0, int e, int step, u32 lc, u32 lr, int4 *next, u32 *ncnt, int *guard,
+                                         u32 *gcnt, bool spec) {
     for (int j = j0; j < e; j += step * KB) {
       int v[KB];
       u64 cs[KB], old[KB], rw[KB];
+      int rs[KB], re[KB];
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         int jj = j + k * step;
@@ -384,23 +409,41 @@ struct Solver {
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? ld_rlx(p.colst + v[k]) : ~0ull;
+      if (spec) {  // narrow level: mate loads ride along with the CAS (one round trip)
 #pragma unroll
-      for (int k = 0; k < KB; k++)  // visited in this GR <=> label carries the current epoch (>= base)
-        old[k] = (v[k] >= 0 && psi_of(cs[k]) < gr_base) ? atomicCAS(p.colst + v[k], cs[k], pack(mu_of(cs[k]), lc))
-                                                         : ~cs[k];
+        for (int k = 0; k < KB; k++) {
+          // unvisited in this GR <=> its label is from an older epoch (< base)
+          const bool try_ = v[k] >= 0 && psi_of(cs[k]) < gr_base;
+          const int w = mu_of(cs[k]);
+          old[k] = try_ ? atomicCAS(p.colst + v[k], cs[k], pack(w, lc)) : ~cs[k];
+          const bool go = try_ && w >= 0;
+          rw[k] = go ? ld_rlx(p.rowst + w) : 0ull;
+          rs[k] = go ? ld_ro(p.rptr + w) : 0;
+          re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
+        }
+      } else {  // wide level: only CAS winners load their mate (no wasted traffic)
 #pragma unroll
-      for (int k = 0; k < KB; k++) {
-        int w = mu_of(cs[k]);
-        rw[k] = (old[k] == cs[k] && w >= 0) ? ld_rlx(p.rowst + w) : 0ull;
+        for (int k = 0; k < KB; k++) {
+          const bool try_ = v[k] >= 0 && psi_of(cs[k]) < gr_base;
+          old[k] = try_ ? atomicCAS(p.colst + v[k], cs[k], pack(mu_of(cs[k]), lc)) : ~cs[k];
+        }
+#pragma unroll
+        for (int k = 0; k < KB; k++) {
+          const int w = mu_of(cs[k]);
+          const bool go = old[k] == cs[k] && w >= 0;
+          rw[k] = go ? ld_rlx(p.rowst + w) : 0ull;
+          rs[k] = go ? ld_ro(p.rptr + w) : 0;
+          re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
+        }
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         if (old[k] != cs[k]) continue;  // not claimed by this thread
         s_grcols++;
         int w = mu_of(cs[k]);
-        if (w >= 0 && mu_of(rw[k]) == v[k]) {
+        if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: mu(v) > -1 and mu(mu(v)) = v
           st_rlx(p.rowst + w, pack(v[k], lr));
-          stage(w, next, ncnt);
+          stage(make_int4(w, rs[k], re[k], 0), next, ncnt);
         } else {
           s_free++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
@@ -415,7 +458,7 @@ struct Solver {
   // guard != nullptr: every reached column that is not matched is appended to
   // guard[0 .. gcount) (the exactness guard, R16).
   template <bool GRID>
-  __device__ int global_relabel(int *&U, int &ulen, int *&T, int *Qa, int *Qb, u32 base, int *guard, int &gcount) {
+  __device__ int global_relabel(int *&U, int &ulen, int *&T, int4 *Qa, int4 *Qb, u32 base, int *guard, int &gcount) {
     GRState g;
     gr_start<GRID>(g, U, ulen, T, Qa, base, guard);
     gr_levels<GRID>(g, base, Qa, Qb, guard, 0x7fffffff);
@@ -430,11 +473,11 @@ struct Solver {
   };
   // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
   template <bool GRID>
-  __device__ void gr_start(GRState &g, int *&U, int &ulen, int *&T, int *Qa, u32 base, int *guard) {
+  __device__ void gr_start(GRState &g, int *&U, int &ulen, int *&T, int4 *Qa, u32 base, int *guard) {
     gr_base = base;
     u32 *gc = &p.ctrl->gcnt;  // zero here: reset one phase after its last use
     trace(1, ulen);
-    gr_level<GRID>(U, ulen, 0, base, Qa, ring_now(0), T, ring_now(1), guard, gc);
+    gr_level<GRID>(U, nullptr, ulen, 0, base, Qa, ring_now(0), T, ring_now(1), guard, gc);
     barrier<GRID>();
     g.nlen = (int)ring_prev(0);
     ulen = (int)ring_prev(1);
@@ -444,16 +487,16 @@ struct Solver {
   // levels 2, 4, ... until the frontier is empty (returns true) or, before expanding
   // a level, the frontier exceeds `limit` (returns false; state kept for resuming).
   template <bool GRID>
-  __device__ bool gr_levels(GRState &g, u32 base, int *Qa, int *Qb, int *guard, int limit) {
+  __device__ bool gr_levels(GRState &g, u32 base, int4 *Qa, int4 *Qb, int *guard, int limit) {
     gr_base = base;
     u32 *gc = &p.ctrl->gcnt;
     while (g.nlen > 0) {
       if (g.nlen > limit) return false;
       g.lvl += 2;
       g.deepest = g.lvl;
-      int *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
+      int4 *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
       trace(2, g.nlen);
-      gr_level<GRID>(cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
+      gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
       barrier<GRID>();
       g.nlen = (int)ring_prev(0);
       g.cur_is_a ^= 1;
@@ -715,75 +758,162 @@ struct Solver {
     return gap == 0x7fffffff ? -1 : gap;
   }
 
-  // ---------------------------------------------------------------- tail mode
-  enum { R_NONE = 0, R_TERM = 1, R_NEEDGR = 2, R_ESC = 3, R_CAP = 4, R_GAP = 5 };
+  // ---------------------------------------------------------------- control state
+  // Alg. 7's control registers.  Every thread holds an identical copy, updated from
+  // values read after barriers; a tail episode publishes the tail group's copy.
+  struct Ctl {
+    long long loop, iterGR, gapAt;
+    int len, ulen;
+    u32 base;
+    int shrink, compact_next, gr_active, ac0, u0, pad;
+    GRState gst;
+    // statistics (meaningful in the lead thread)
+    long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop;
+  };
+  static_assert(sizeof(Ctl) % 8 == 0 && sizeof(Ctl) / 8 <= 32, "Ctl handoff image");
+  __device__ __forceinline__ int *Acp(const Ctl &c) const { return c.ac0 ? p.wl0 : p.wl1; }
+  __device__ __forceinline__ int *App(const Ctl &c) const { return c.ac0 ? p.wl1 : p.wl0; }
+  __device__ __forceinline__ int *Ub(const Ctl &c) const { return c.u0 ? p.qa : p.qb; }
+  __device__ __forceinline__ int *Tb(const Ctl &c) const { return c.u0 ? p.qb : p.qa; }
+  __device__ __forceinline__ u32 stride() const { return (u32)(m + n + 2); }
+  __device__ __forceinline__ int4 *Q4(int i) const { return reinterpret_cast<int4 *>(i ? p.qd : p.qc); }
+  __device__ __forceinline__ bool base_overflow(const Ctl &c) const {
+    return (u64)c.base + 2ull * stride() >= 0xfffffff0ull;
+  }
+
+  enum { R_NONE = 0, R_TERM = 1, R_GRID = 2, R_CAP = 4 };
   // gap relabel schedule (R14): once, halfway between two GRs
   __device__ __forceinline__ long long gap_at(long long loop, long long iterGR) const {
     return (p.gap && iterGR - loop >= 2) ? loop + (iterGR - loop) / 2 : -1;
   }
-  __device__ __forceinline__ int tail_f() const { return p.tail_max * 2; }
+  // GR frontiers of at most tail_f() rows run on the tail group (hand-over back to
+  // the grid when a frontier outgrows it, back to the tail below tail_f()/2)
+  __device__ __forceinline__ int tail_f() const { return p.tail_f > 0 ? p.tail_f : 2 * p.tail_max; }
 
-  // All CTAs call.  CTA 0 runs Alg. 7 iterations alone -- fix with compaction at
-  // every step, push, and GRs whose frontiers stay narrow -- with __syncthreads
-  // between phases, while the other CTAs wait at one grid barrier.  The episode
-  // ends when a GR needs the grid (too many unmatched rows, or a frontier that
-  // grew past tail_f(): R_ESC hands the BFS state over), when no active column is
-  // left (R_TERM) or at the iteration cap (R_CAP).  CTA 0 then publishes its
-  // control registers and every CTA adopts them after the barrier.
-  __device__ int tail_episode(long long &loop, long long &iterGR, long long &gapAt, int &len, int &ulen, u32 &base,
-                              bool &shrink,
-                              int *&Ac, int *&Ap, int *&U, int *&T, int *Qa, int *Qb, GRState &gst, long long &grs,
-                              long long &levels, long long &shrinks, long long &tail_loops, long long &ns_gr,
-                              long long &ns_loop) {
-    const u32 stride = (u32)(m + n + 2);
-    int reason = R_NONE;
-    Ctrl *c = p.ctrl;
-    if (blockIdx.x < p.tail_ctas) {
-      const int limit = tail_f();
-      for (;;) {
-        if (loop >= p.max_loops) { reason = R_CAP; break; }
-        if (loop == gapAt) { reason = R_GAP; break; }
-        if (loop == iterGR) {
-          if (ulen > limit || (u64)base + 2ull * stride >= 0xfffffff0ull) { reason = R_NEEDGR; break; }
-          u64 g0 = gtime();
-          gr_start<false>(gst, U, ulen, T, Qa, base, nullptr);
-          bool done = gr_levels<false>(gst, base, Qa, Qb, nullptr, limit);
-          ns_gr += (long long)(gtime() - g0);
-          if (!done) { reason = R_ESC; break; }
-          int ml = gst.deepest + 2;
-          grs++; levels += ml / 2;
-          iterGR = loop + iter_gap(ml);
-          gapAt = gap_at(loop, iterGR);
-          shrink = true;
-          base += stride;
-        }
-        u64 l0 = gtime();
-        const int lp = (int)loop;
-        if (threadIdx.x == 0) s_slots += len;
-        trace(3, len);
-        int r1 = compact_pass1<false>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
-        barrier<false>();
-        if (p.tail_ctas > 1) {
-          len = compact_pass2<false>(len, T, Ac, r1);
-          barrier<false>();
-        } else {
-          len = r1;
-        }
-        if (shrink) { shrinks++; shrink = false; }
-        if (len == 0) { reason = R_TERM; ns_loop += (long long)(gtime() - l0); break; }
-        trace(4, len);
-        push<false>(len, Ac, Ap, lp, base - stride);
-        barrier<false>();
-        int *tmp = Ac; Ac = Ap; Ap = tmp;
-        loop++;
-        tail_loops++;
-        ns_loop += (long long)(gtime() - l0);
+  // ---------------------------------------------------------------- units of work
+  // GR bookkeeping once the BFS is over (Alg. 7 l.7-9 with GETITERGR, R7)
+  __device__ void gr_finish(Ctl &c) {
+    int ml = c.gst.deepest + 2;
+    c.grs++;
+    c.levels += ml / 2;
+    c.iterGR = c.loop + iter_gap(ml);
+    c.gapAt = gap_at(c.loop, c.iterGR);
+    c.shrink = 1;
+    c.gr_active = 0;
+    c.base += stride();
+  }
+  // GR level 0 (INITRELABEL via the epoch bump + first expansion)
+  template <bool GRID>
+  __device__ void gr_begin(Ctl &c) {
+    u64 g0 = gtime();
+    int *U = Ub(c), *T = Tb(c);
+    gr_start<GRID>(c.gst, U, c.ulen, T, Q4(0), c.base, nullptr);
+    c.u0 ^= 1;
+    c.gr_active = 1;
+    if (c.gst.nlen == 0) gr_finish(c);
+    c.ns_gr += (long long)(gtime() - g0);
+  }
+  // one BFS level (Alg. 5)
+  template <bool GRID>
+  __device__ void gr_step(Ctl &c) {
+    u64 g0 = gtime();
+    GRState &g = c.gst;
+    g.lvl += 2;
+    g.deepest = g.lvl;
+    int4 *cur = Q4(g.cur_is_a ? 0 : 1), *nxt = Q4(g.cur_is_a ? 1 : 0);
+    gr_base = c.base;
+    trace(2, g.nlen);
+    gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
+    barrier<GRID>();
+    g.nlen = (int)ring_prev(0);
+    g.cur_is_a ^= 1;
+    if (g.nlen == 0) gr_finish(c);
+    c.ns_gr += (long long)(gtime() - g0);
+  }
+  // one iteration of Alg. 7 l.10-19: fix step (INITKRNL, or SHRKRNL = fix + stable
+  // compaction), then PUSHKRNL and the Ac/Ap swap.  Returns false when the fix
+  // step found no active column.  The tail group compacts at every step.
+  template <bool GRID>
+  __device__ bool loop_step(Ctl &c) {
+    u64 l0 = gtime();
+    const u32 cur = c.base - stride();  // epoch of the labels in use
+    int *Ac = Acp(c), *Ap = App(c);
+    const int lp = (int)c.loop;
+    int act;
+    trace(3, c.len);
+    if (!GRID || (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) || p.compact_every || c.compact_next) {
+      if (threadIdx.x == 0 && (GRID ? blockIdx.x == 0 : true)) s_slots += c.len;
+      int r1 = compact_pass1<GRID>(c.len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, Tb(c), Ac);
+      barrier<GRID>();
+      if (ncta<GRID>() > 1) {
+        c.len = compact_pass2<GRID>(c.len, Tb(c), Ac, r1);
+        barrier<GRID>();  // Ac was rewritten by other CTAs: order it before PUSH
+      } else {
+        c.len = r1;
       }
-      if (threadIdx.x == 0) {
-        c->ho_reason = reason; c->ho_ph = ph; c->ho_len = len; c->ho_ulen = ulen; c->ho_shrink = shrink;
-        c->ho_ac0 = (Ac == p.wl0); c->ho_u0 = (U == p.qa); c->ho_loop = loop; c->ho_iter = iterGR;
-        c->ho_base = base; c->ho_gapat = gapAt; c->ho_gl = gst.lvl; c->ho_gd = gst.deepest; c->ho_gn = gst.nlen; c->ho_gc = gst.cur_is_a;
-        for (int j = 0; j < 4; j++) c->ring[j][0] = c->ring[j][1] = c->ring[j][2] = c->ring[j][3] = 0;
+      act = c.len;
+      if (c.shrink) c.shrinks++;
+      c.shrink = 0;
+      c.compact_next = 0;
+    } else {
+      fix_plain<true>(c.len, Ac, Ap, lp, 0);
+      barrier<true>();
+      act = (int)ring_prev(0);
+      // adaptive compaction (beyond the paper's post-GR shrink): when most slots
+      // are empty the next fix step compacts, so the tail group can take over
+      if (p.compact_adapt && act > 0 && (long long)act * 4 < c.len && c.len > p.tail_max) c.compact_next = 1;
+    }
+    debug_check(3, c.loop, Ac, c.len);
+    if (act == 0) {
+      c.ns_loop += (long long)(gtime() - l0);
+      return false;
+    }
+    trace(4, c.len);
+    push<GRID>(c.len, Ac, Ap, lp, cur);
+    barrier<GRID>();
+    debug_check(4, c.loop, nullptr, 0);
+    c.ac0 ^= 1;  // l.18: swap Ac and Ap
+    c.loop++;    // l.19
+    if (GRID) c.loops++; else c.tail_loops++;
+    c.ns_loop += (long long)(gtime() - l0);
+    return true;
+  }
+
+  // ---------------------------------------------------------------- tail mode
+  // All CTAs call.  The tail group (CTA 0, or cluster 0) runs units of work alone
+  // with CTA (cluster) barriers -- fix/push loops on worklists of at most tail_max
+  // slots, GR levels of at most tail_f() rows -- while the other CTAs wait at one
+  // grid barrier; most of the paper's iterations have "only a few" active columns
+  // (P:525-528).  It stops when a unit needs the grid (R_GRID), when no active
+  // column is left (R_TERM) or at the iteration cap (R_CAP), publishes its Ctl and
+  // every CTA adopts it after the barrier.
+  __device__ int tail_episode(Ctl &c) {
+    int reason = R_NONE;
+    Ctrl *x = p.ctrl;
+    if (blockIdx.x < p.tail_ctas) {
+      const int up = tail_f();
+      for (;;) {
+        if (c.loop >= p.max_loops) { reason = R_CAP; break; }
+        if (c.gr_active) {
+          if (c.gst.nlen > up) { reason = R_GRID; break; }
+          gr_step<false>(c);
+          continue;
+        }
+        if (c.loop == c.gapAt) { reason = R_GRID; break; }
+        if (c.loop == c.iterGR) {
+          if (c.ulen > up || base_overflow(c)) { reason = R_GRID; break; }
+          gr_begin<false>(c);
+          continue;
+        }
+        if (c.len > p.tail_max) { reason = R_GRID; break; }
+        if (!loop_step<false>(c)) { reason = R_TERM; break; }
+      }
+      if (threadIdx.x == 0 && blockIdx.x == 0) {
+        x->ho_reason = reason;
+        x->ho_ph = ph;
+        const long long *src = reinterpret_cast<const long long *>(&c);
+        for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) x->ho[j] = src[j];
+        for (int j = 0; j < 4; j++) x->ring[j][0] = x->ring[j][1] = x->ring[j][2] = x->ring[j][3] = 0;
       }
     }
     if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
@@ -792,31 +922,54 @@ struct Solver {
     }
     grid_sync(&p.ctrl->bar, true);
     nbar++;
-    reason = ld_rlx((const u32 *)&c->ho_reason);
-    ph = (int)ld_rlx((const u32 *)&c->ho_ph) + 1;
-    len = (int)ld_rlx((const u32 *)&c->ho_len);
-    ulen = (int)ld_rlx((const u32 *)&c->ho_ulen);
-    shrink = ld_rlx((const u32 *)&c->ho_shrink) != 0;
-    bool ac0 = ld_rlx((const u32 *)&c->ho_ac0) != 0, u0 = ld_rlx((const u32 *)&c->ho_u0) != 0;
-    Ac = ac0 ? p.wl0 : p.wl1; Ap = ac0 ? p.wl1 : p.wl0;
-    U = u0 ? p.qa : p.qb; T = u0 ? p.qb : p.qa;
-    loop = ld_rlx(&c->ho_loop);
-    iterGR = ld_rlx(&c->ho_iter);
-    gapAt = ld_rlx(&c->ho_gapat);
-    base = ld_rlx(&c->ho_base);
-    gst.lvl = (int)ld_rlx((const u32 *)&c->ho_gl); gst.deepest = (int)ld_rlx((const u32 *)&c->ho_gd);
-    gst.nlen = (int)ld_rlx((const u32 *)&c->ho_gn); gst.cur_is_a = (int)ld_rlx((const u32 *)&c->ho_gc);
+    reason = (int)ld_rlx((const u32 *)&x->ho_reason);
+    ph = (int)ld_rlx((const u32 *)&x->ho_ph) + 1;
+    long long *dst = reinterpret_cast<long long *>(&c);
+    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) dst[j] = ld_rlx(&x->ho[j]);
     return reason;
+  }
+
+  // exactness guard (R16): one more GR; every unmatched column it reaches is
+  // re-activated and the loop resumes (returns true); otherwise the labels certify
+  // maximality (returns false).
+  __device__ bool guard_step(Ctl &c) {
+    if (!p.final_check) return false;
+    u64 g0 = gtime();
+    if (base_overflow(c)) { reset_labels(); c.base = 1; }
+    int gcount = 0;
+    int *Ac = Acp(c), *Ap = App(c);
+    int *U = Ub(c), *T = Tb(c);
+    int ml = global_relabel<true>(U, c.ulen, T, Q4(0), Q4(1), c.base, Ac, gcount);
+    c.u0 ^= 1;
+    c.grs++;
+    c.levels += ml / 2;
+    c.base += stride();
+    c.ns_gr += (long long)(gtime() - g0);
+    if (gcount == 0) return false;
+    c.guard_re += gcount;
+    for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
+      int v = __ldcg(Ac + i);
+      u64 cs = ld_rlx(p.colst + v);
+      st_rlx(p.colst + v, pack(-1, psi_of(cs)));
+      Ap[i] = v;
+    }
+    barrier<true>();
+    if (blockIdx.x == 0 && threadIdx.x == 0) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
+    c.len = gcount;
+    c.iterGR = c.loop + iter_gap(ml);
+    c.gapAt = gap_at(c.loop, c.iterGR);
+    c.shrink = 0;
+    return true;
   }
 
   // ---------------------------------------------------------------- the solve
   __device__ void run() {
     const bool lead = blockIdx.x == 0 && threadIdx.x == 0;
     u64 t0 = gtime(), tA = t0;
-    long long ns_gr = 0, ns_loop = 0, ns_init = 0;
-    long long grs = 0, levels = 0, shrinks = 0, loops = 0, guard_re = 0;
+    long long ns_init = 0;
     int *Ac = p.wl0, *Ap = p.wl1;
-    int *U = p.qa, *T = p.qb, *Qa = p.qc, *Qb = p.qd;
+    int *U = p.qa, *T = p.qb;
+    int4 *Qa = Q4(0), *Qb = Q4(1);
     if (threadIdx.x == 0) sm.qcnt = 0;
     init_state();
     barrier<true>();
@@ -832,8 +985,6 @@ struct Solver {
     int ulen = (int)ring_prev(0);
     int len = compact_pass2<true>(n, T, Ac, run1, Ap);  // Ap = Ac (R12)
     long long init_card = (long long)m - ulen;
-    u32 base = 1;  // epoch of the next GR
-    const u32 stride = (u32)(m + n + 2);
 
     if (p.mode == MODE_GAP) {  // mcm_gap_relabel: labels in, labels out
       int gl = gap_relabel(1);
@@ -844,144 +995,69 @@ struct Solver {
     }
     if (p.mode == MODE_RELABEL) {
       int g;
-      int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, nullptr, g);
-      write_labels(base);
-      if (lead) {
-        p.ctrl->stat[ST_MAXLEVEL] = ml;
-      }
+      int ml = global_relabel<true>(U, ulen, T, Qa, Qb, 1, nullptr, g);
+      write_labels(1);
+      if (lead) p.ctrl->stat[ST_MAXLEVEL] = ml;
       finish_stats(0, 0, 0, 0, 0, 0, 0, 0, 0, 0, 0);
       return;
     }
 
     barrier<true>();
     debug_check(2, -1, Ac, len);
-    u64 t1 = gtime();
-    ns_init = (long long)(t1 - t0);
+    ns_init = (long long)(gtime() - t0);
 
-    long long loop = 0, iterGR = 0, tail_loops = 0, gapAt = -1, gaps = 0;
-    bool shrink = false, compact_next = false;
-    GRState gst;
-    int reason = R_NONE;
+    Ctl c;
+    memset(&c, 0, sizeof(c));
+    c.len = len; c.ulen = ulen; c.base = 1; c.gapAt = -1; c.ac0 = 1; c.u0 = 1;  // loop = iterGR = 0
     for (;;) {
-      if (loop >= p.max_loops) {
+      if (c.loop >= p.max_loops) {
         if (lead) p.ctrl->err = -5;
         break;
       }
-      bool terminated = false;
-      reason = R_NONE;
-      // ---- tail episode: a short worklist runs on CTA 0 alone (CTA barriers)
-      if (p.tail_max > 0 && len <= p.tail_max && !(loop == iterGR && ulen > tail_f())) {
-        reason = tail_episode(loop, iterGR, gapAt, len, ulen, base, shrink, Ac, Ap, U, T, Qa, Qb, gst, grs, levels,
-                              shrinks, tail_loops, ns_gr, ns_loop);
-        if (reason == R_CAP) {
+      const int up = tail_f();
+      bool tail_ok = p.tail_max > 0 &&
+                     (c.gr_active ? c.gst.nlen <= up / 2
+                                  : (c.loop == c.gapAt ? false
+                                                       : (c.loop == c.iterGR ? (c.ulen <= up && !base_overflow(c))
+                                                                             : c.len <= p.tail_max)));
+      if (tail_ok) {
+        int r = tail_episode(c);
+        if (r == R_CAP) {
           if (lead) p.ctrl->err = -5;
           break;
         }
-        if (reason == R_TERM) terminated = true;
+        if (r == R_TERM && !guard_step(c)) break;
+        continue;
       }
-      if (!terminated && loop == gapAt) {                              // gap relabel (R14)
+      // one unit of grid work
+      if (c.gr_active) { gr_step<true>(c); continue; }                // Alg. 5 level
+      if (c.loop == c.gapAt) {                                         // gap relabel (R14)
         u64 g0 = gtime();
-        if (gap_relabel(base - stride) >= 0) gaps++;
-        gapAt = -1;
-        ns_gr += (long long)(gtime() - g0);
-        if (p.tail_max > 0 && len <= p.tail_max && loop != iterGR) continue;
+        if (gap_relabel(c.base - stride()) >= 0) c.gaps++;
+        c.gapAt = -1;
+        c.ns_gr += (long long)(gtime() - g0);
+        continue;
       }
-      if (!terminated) {
-        if (reason == R_ESC || loop == iterGR) {                       // Alg. 7 l.6
-          u64 g0 = gtime();
-          int ml;
-          if (reason == R_ESC) {  // a tail GR whose frontier grew too wide: finish it here
-            gr_levels<true>(gst, base, Qa, Qb, nullptr, 0x7fffffff);
-            ml = gst.deepest + 2;
-          } else {
-            if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
-            int gdummy;
-            ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, nullptr, gdummy);   // l.7
-          }
-          grs++; levels += ml / 2;
-          iterGR = loop + iter_gap(ml);                                // l.8
-          gapAt = gap_at(loop, iterGR);
-          shrink = true;                                               // l.9
-          base += stride;
-          ns_gr += (long long)(gtime() - g0);
-          if (p.tail_max > 0 && len <= p.tail_max) continue;           // fix + push in the tail
-        }
-        const u32 cur = base - stride;  // epoch of the labels in use
-        u64 l0 = gtime();
-        int act;
-        if ((shrink && p.shrink_min >= 0 && len >= p.shrink_min) || p.compact_every || compact_next) {  // l.11
-          const int lp = (int)loop;
-          int r1 = compact_pass1<true>(len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, T, Ac);
-          s_slots += 0;
-          if (lead) s_slots += len;
-          barrier<true>();
-          len = compact_pass2<true>(len, T, Ac, r1);                   // SHRKRNL
-          act = len;
-          if (shrink) shrinks++;
-          shrink = false;                                              // l.13
-          compact_next = false;
-          // Ac was rewritten by CTAs other than the pushing one: order it before PUSH
-          barrier<true>();
-        } else {
-          trace(3, len);
-          fix_plain<true>(len, Ac, Ap, (int)loop, 0);                  // l.15
-          barrier<true>();
-          act = (int)ring_prev(0);
-          // adaptive compaction (beyond the paper's post-GR shrink): when most slots
-          // are empty, the next fix step compacts, so the tail group can take over
-          if (p.compact_adapt && act > 0 && (long long)act * 4 < len && len > p.tail_max) compact_next = true;
-        }
-        debug_check(3, loop, Ac, len);
-        if (act != 0) {
-          trace(4, len);
-          push<true>(len, Ac, Ap, (int)loop, cur);                     // l.17
-          barrier<true>();
-          debug_check(4, loop, nullptr, 0);
-          int *tmp = Ac; Ac = Ap; Ap = tmp;                            // l.18
-          loop++;                                                      // l.19
-          loops++;
-          ns_loop += (long long)(gtime() - l0);
-          continue;
-        }
-        ns_loop += (long long)(gtime() - l0);
+      if (c.loop == c.iterGR) {                                        // Alg. 7 l.6-9
+        if (base_overflow(c)) { reset_labels(); c.base = 1; }
+        gr_begin<true>(c);
+        continue;
       }
-      // ---- no active column left (l.5 / l.16)
-      if (!p.final_check) break;
-      // exactness guard (R16): one more GR; every unmatched column it reaches is
-      // re-activated and the loop resumes; otherwise psi certifies maximality.
-      u64 g0 = gtime();
-      if ((u64)base + 2ull * stride >= 0xfffffff0ull) { reset_labels(); base = 1; }
-      int gcount = 0;
-      int ml = global_relabel<true>(U, ulen, T, Qa, Qb, base, Ac, gcount);
-      grs++; levels += ml / 2;
-      base += stride;
-      ns_gr += (long long)(gtime() - g0);
-      if (gcount == 0) break;
-      guard_re += gcount;
-      for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
-        int v = __ldcg(Ac + i);
-        u64 cs = ld_rlx(p.colst + v);
-        st_rlx(p.colst + v, pack(-1, psi_of(cs)));
-        Ap[i] = v;
-      }
-      barrier<true>();
-      if (lead) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
-      len = gcount;
-      iterGR = loop + iter_gap(ml);
-      gapAt = gap_at(loop, iterGR);
-      shrink = false;
+      if (!loop_step<true>(c) && !guard_step(c)) break;               // l.10-19 / termination
     }
-    loops += tail_loops;
-    gaps_total = gaps;
+    gaps_total = c.gaps;
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
-    finish_stats(loops, grs, levels, shrinks, guard_re, init_card, ns_init, ns_gr, ns_loop, (long long)(gtime() - tA),
-                 tail_loops);
+    finish_stats(c.loops + c.tail_loops, c.grs, c.levels, c.shrinks, c.guard_re, init_card, ns_init, c.ns_gr,
+                 c.ns_loop, (long long)(gtime() - tA), c.tail_loops);
   }
 
   __device__ void reset_labels() {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
-    for (int u = g; u < m; u += G) { u64 w = ld_rlx(p.rowst + u); st_rlx(p.rowst + u, pack(mu_of(w), 0)); }
+    for (int u = g; u < m; u += G) {
+      u64 w = ld_rlx(p.rowst + u);
+      st_rlx(p.rowst + u, pack(mu_of(w), 0));
+    }
     for (int v = g; v < n; v += G) { u64 w = ld_rlx(p.colst + v); st_rlx(p.colst + v, pack(mu_of(w), 0)); }
     barrier<true>();
   }
@@ -1016,7 +1092,8 @@ struct Solver {
 #define MCM_MINB 1
 #endif
 __global__ void __launch_bounds__(NT, MCM_MINB) gpr_kernel(Params p) {
-  __shared__ Smem sm;
+  extern __shared__ __align__(16) unsigned char smem_raw[];
+  Smem &sm = *reinterpret_cast<Smem *>(smem_raw);
   Solver s(p, sm);
   s.run();
 }
