@@ -193,8 +193,8 @@ void mcm_default_options(mcm_options_t *o) {
   o->gap = 0;
   o->final_check = 1;
   o->dead_skip = 1;
-  o->tail_max = 512;
-  o->tail_f = 0;
+  o->tail_max = 256;
+  o->tail_f = 128;
   o->tail_ctas = 1;
   o->compact_adapt = 1;
   o->compact_every = 0;

@@ -23,8 +23,13 @@ constexpr int NT = 512;          // threads per CTA
 constexpr int NWARP = NT / 32;
 constexpr int QCAP = 16384;      // shared staging (ints, 64 KB, dynamic smem): next BFS frontier, gap histogram
 constexpr int QCAP4 = QCAP / 4;  // ... as int4 frontier entries
+constexpr int TQ = QCAP4 / 2;    // tail: two shared int4 frontier buffers of TQ entries (alias q)
+constexpr int TW = 1024;         // tail: shared worklist capacity (Ac / Ap)
 constexpr int SMALL_DEG = 32;    // greedy: adjacency lists up to this length: one thread
 constexpr int BIG_DEG = 64;      // GR / push: longer lists go to the whole warp
+constexpr int HUGE_DEG = 512;    // push: longer lists go to the whole CTA
+constexpr int MAXHUGE = 32;      // CTA-wide push list per tile
+constexpr int HUGE_CTA = 4;      // at most this many per tile: one CTA-wide scan each; more: a warp each
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
 
 enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
@@ -79,14 +84,25 @@ struct Smem {
   long long red[NWARP];
   int w[NWARP];
   alignas(16) int q[QCAP];
+  int wl[2][TW];           // tail: the worklist (Ac/Ap) while the single-CTA tail owns it
+  int4 huge[MAXHUGE];      // push: columns deferred to the CTA-wide scan {slot, v, s, e}
+  u64 hugec[MAXHUGE];
+  int huget[MAXHUGE];
+  int nhuge;
   int qcnt, qbase, tmp;
 };
+
+// worklist / frontier loads: shared (tail residency) or global (bypass L1)
+__device__ __forceinline__ int ld_wl(const int *p) { return __isShared(p) ? *p : __ldcg(p); }
+__device__ __forceinline__ int4 ld_q(const int4 *p) { return __isShared(p) ? *p : __ldcg(p); }
 
 __device__ __forceinline__ u64 gtime() {
   u64 t;
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
 }
+// phase timers: only the lead thread (block 0, thread 0) reads the clock
+__device__ __forceinline__ u64 tnow() { return (threadIdx.x == 0 && blockIdx.x == 0) ? gtime() : 0ull; }
 
 struct Solver {
   const Params &p;
@@ -102,6 +118,13 @@ struct Solver {
   __device__ __forceinline__ void trace(int tag, int sz) {
     ttag = tag; tsz = sz;
   }
+  // extra trace point (no barrier): lead thread only
+  __device__ __forceinline__ void tmark(int tag, int sz) {
+    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
+      p.trace[3 * tn] = tag; p.trace[3 * tn + 1] = sz; p.trace[3 * tn + 2] = (long long)gtime();
+      tn++;
+    }
+  }
 
   __device__ Solver(const Params &p_, Smem &sm_) : p(p_), sm(sm_), m(p_.m), n(p_.n), INF(p_.m + p_.n) {}
 
@@ -111,10 +134,6 @@ struct Solver {
   // and consumed at the start of the previous phase, so CTA 0 may clear it now.
   template <bool GRID>
   __device__ __forceinline__ void barrier() {
-    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
-      p.trace[3 * tn] = ttag * 2 + (GRID ? 1 : 0); p.trace[3 * tn + 1] = tsz; p.trace[3 * tn + 2] = (long long)gtime();
-      tn++;
-    }
     if (GRID) {
       grid_sync(&p.ctrl->bar, false);
       nbar++;
@@ -124,6 +143,12 @@ struct Solver {
       asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
     } else {
       __syncthreads();
+    }
+    // phase trace: stamped after the barrier, so a phase's duration includes its
+    // slowest CTA
+    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
+      p.trace[3 * tn] = ttag * 2 + (GRID ? 1 : 0); p.trace[3 * tn + 1] = tsz; p.trace[3 * tn + 2] = (long long)gtime();
+      tn++;
     }
     ph++;
     if (blockIdx.x == 0 && threadIdx.x == 0) {
@@ -164,8 +189,8 @@ struct Solver {
     if (g.thread_rank() == 0) base = atomicAdd(&sm.qcnt, (int)g.size());
     base = g.shfl(base, 0);
     int q = base + (int)g.thread_rank();
-    if (q < QCAP4) {
-      reinterpret_cast<int4 *>(sm.q)[q] = x;
+    if (q < (sq ? TQ : QCAP4)) {
+      (sq ? sq_next : reinterpret_cast<int4 *>(sm.q))[q] = x;
     } else {  // overflow: direct append, again one global atomic per group
       cg::coalesced_group o = cg::coalesced_threads();
       u32 gb = 0;
@@ -175,6 +200,7 @@ struct Solver {
     }
   }
   __device__ __forceinline__ void flush(int4 *next, u32 *gcnt) {
+    if (sq) return;  // tail: the next frontier is the shared buffer itself
     __syncthreads();
     int c = min(sm.qcnt, QCAP4);
     if (threadIdx.x == 0) sm.qbase = c ? (int)atomicAdd(gcnt, (u32)c) : 0;
@@ -375,7 +401,7 @@ struct Solver {
         if (keep) Uout[sm.tmp + r] = u;
         if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
       } else if (i < curlen) {
-        int4 q = __ldcg(cur4 + i);
+        int4 q = ld_q(cur4 + i);
         u = q.x; s = q.y; e = q.z;
       }
       if (u >= 0 && gl == 0) { s_grrows++; s_gredges += e - s; }
@@ -452,6 +478,9 @@ struct Solver {
     }
   }
   u32 gr_base = 0;
+  bool sq = false;          // tail GR: stage() writes straight into sq_next (shared)
+  int4 *sq_next = nullptr;
+  __device__ __forceinline__ int4 *sfr(int i) { return reinterpret_cast<int4 *>(sm.q) + i * TQ; }
 
   // Full GR (Alg. 4).  U/T: unmatched-row list and a free buffer
   // (swapped on return); Qa/Qb frontier buffers.  Returns maxLevel.
@@ -469,7 +498,7 @@ struct Solver {
   // The GR as a resumable state machine, so that a CTA-local GR (tail mode) can
   // hand a frontier that grew too wide over to the whole grid mid-BFS.
   struct GRState {
-    int lvl, deepest, nlen, cur_is_a;
+    int lvl, deepest, nlen, cur_is_a, in_smem, pad;
   };
   // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
   template <bool GRID>
@@ -509,13 +538,13 @@ struct Solver {
   // race (Ap(i) = v still unmatched => Ac(i) <- v, l.3-6), then mark the slot's
   // column active in this loop (l.8-11, reading R5: after the if/else).
   __device__ __forceinline__ int fix_slot(int i, int *Ac, const int *Ap, int loop) {
-    int v = ld_cg(Ap + i);
+    int v = ld_wl(Ap + i);
     int a;
     if (v != -1 && col_unmatched(v)) {
       Ac[i] = v;
       a = v;
     } else {
-      a = ld_cg(Ac + i);
+      a = ld_wl(Ac + i);
     }
     if (a != -1) st_rlx(p.iA + a, loop);
     return a;
@@ -533,10 +562,32 @@ struct Solver {
   }
 
   // ---------------------------------------------------------------- push
-  // G-PR-PUSHKRNL (Alg. 9) over slots [0, len).  Columns with short
-  // lists scan alone; longer lists are scanned by the whole warp in chunks of 32
-  // with a (label, position) min-reduction and the early exit at psi(v)-1 taken
-  // per chunk (reading R11).
+  // G-PR-PUSHKRNL (Alg. 9) over slots [0, len).  Each column gets a lane
+  // group (pick_group); lists longer than BIG_DEG go to the whole warp, lists longer
+  // than HUGE_DEG to the whole CTA (a straggler column would otherwise hold up the
+  // phase: C2's dense "rail" columns have 2,000 rows).  Every scan takes a
+  // (label, position) minimum per step with the early exit at psi(v)-1 (R11).
+  __device__ __forceinline__ void push_finalize(int i, int v, u64 cs, u64 best, int ub, int wb, int loop, u32 base,
+                                                int *Ac, int *Ap) {
+    int psimin = best == ~0ull ? INF : (int)(best >> 32);
+    if (psimin < INF) {                                 // l.12
+      if (wb == -1 || ld_rlx(p.iA + wb) != loop) {      // l.13
+        st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
+        st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
+        Ap[i] = wb;                                     // l.18 (R3)
+        s_push++;
+      } else {
+        Ap[i] = -1;                                     // R4: blocked
+        s_block++;
+      }
+    } else {
+      st_rlx(p.colst + v, pack(-2, psi_of(cs)));        // l.20
+      Ac[i] = -1;                                       // l.21
+      Ap[i] = -1;                                       // l.22
+      s_dead++;
+    }
+  }
+
   template <bool GRID>
   __device__ void push(int len, int *Ac, int *Ap, int loop, u32 base) {
     const int lane = lane_id();
@@ -545,7 +596,7 @@ struct Solver {
     const unsigned gmask = group_mask(G);
     for (int t = cta<GRID>() * per_tile; t < len; t += ncta<GRID>() * per_tile) {
       int i = t + (int)threadIdx.x / G;
-      int v = (i < len) ? ld_cg(Ac + i) : -1;
+      int v = (i < len) ? ld_wl(Ac + i) : -1;
       int s = 0, e = 0, psiv = INF;
       u64 cs = 0;
       if (v >= 0) {
@@ -556,10 +607,17 @@ struct Solver {
         if (p.dead_skip && psiv >= INF) e = s;  // R19: provably unmatchable
       }
       const int target = psiv - 1;
-      const bool big = v >= 0 && G < 32 && e - s > BIG_DEG;
+      bool huge = v >= 0 && e - s > HUGE_DEG;
+      if (huge && gl == 0) {  // defer to the CTA-wide pass below
+        int q = atomicAdd(&sm.nhuge, 1);
+        if (q < MAXHUGE) { sm.huge[q] = make_int4(i, v, s, e); sm.hugec[q] = cs; sm.huget[q] = target; }
+        else huge = false;  // list full: the warp takes it
+      }
+      huge = __shfl_sync(gmask, huge, lane & ~(G - 1));
+      const bool big = v >= 0 && !huge && G < 32 && e - s > BIG_DEG;
       u64 best = ~0ull;
       int ub = -1, wb = -1;
-      if (v >= 0 && !big) scan(s, e, gl, G, gmask, target, base, best, ub, wb);      // l.6-11
+      if (v >= 0 && !big && !huge) scan(s, e, gl, G, gmask, target, base, best, ub, wb);  // l.6-11
       unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
       while (bigm) {  // long lists: the whole warp
         int bl = __ffs(bigm) - 1;
@@ -571,29 +629,82 @@ struct Solver {
         scan(sb, eb, lane, 32, 0xffffffffu, tb, base, b2, u2, w2);
         if (lane == bl) { best = b2; ub = u2; wb = w2; }
       }
-      if (gl != 0) continue;
-      if (v >= 0) {
-        int psimin = best == ~0ull ? INF : (int)(best >> 32);
-        if (psimin < INF) {                                 // l.12
-          if (wb == -1 || ld_rlx(p.iA + wb) != loop) {      // l.13
-            st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
-            st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
-            Ap[i] = wb;                                     // l.18 (R3)
-            s_push++;
-          } else {
-            Ap[i] = -1;                                     // R4: blocked
-            s_block++;
-          }
-        } else {
-          st_rlx(p.colst + v, pack(-2, psi_of(cs)));        // l.20
-          Ac[i] = -1;                                       // l.21
-          Ap[i] = -1;                                       // l.22
-          s_dead++;
-        }
-      } else if (i < len) {
-        Ap[i] = -1;                                         // l.24
+      if (gl == 0 && !huge) {
+        if (v >= 0) push_finalize(i, v, cs, best, ub, wb, loop, base, Ac, Ap);
+        else if (i < len) Ap[i] = -1;                   // l.24
       }
+      __syncthreads();
+      const int nh = min(sm.nhuge, MAXHUGE);
+      if (nh <= HUGE_CTA) {
+        for (int h = 0; h < nh; h++) {  // a few very long lists: the whole CTA each
+          const int4 hq = sm.huge[h];
+          u64 hb;
+          int hu, hw;
+          scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
+          if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+        }
+      } else {
+        for (int h = warp_id(); h < nh; h += NWARP) {  // many: one warp each, in parallel
+          const int4 hq = sm.huge[h];
+          u64 hb;
+          int hu, hw;
+          scan(hq.z, hq.w, lane, 32, 0xffffffffu, sm.huget[h], base, hb, hu, hw);
+          if (lane == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+        }
+      }
+      __syncthreads();
+      if (threadIdx.x == 0) sm.nhuge = 0;
+      __syncthreads();
     }
+  }
+  // scan() with the whole CTA: KB*NT neighbours per step; CTA-wide (label, position)
+  // minimum through shared memory; returns the result in every thread.
+  __device__ void scan_cta(int s, int e, int target, u32 base, u64 &best, int &bu, int &bw) {
+    best = ~0ull;
+    bu = -1;
+    bw = -1;
+    for (int c0 = s; c0 < e; c0 += NT * KB) {
+      int x[KB];
+      u64 rs[KB];
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        int jj = c0 + (int)threadIdx.x + k * NT;
+        x[k] = jj < e ? ld_ro(p.cadj + jj) : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+      u64 key = ~0ull;
+      int kx = -1, kw = -1;
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        if (x[k] < 0) continue;
+        s_scan++;
+        int l = lab(psi_of(rs[k]), base, INF);
+        u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + (int)threadIdx.x + k * NT - s)) : ~0ull;
+        if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
+      }
+      u64 km = key;
+#pragma unroll
+      for (int o = 16; o > 0; o >>= 1) {
+        u64 other = __shfl_xor_sync(0xffffffffu, km, o);
+        km = other < km ? other : km;
+      }
+      __syncthreads();
+      if (lane_id() == 0) sm.red[warp_id()] = (long long)km;
+      __syncthreads();
+      u64 kmin = ~0ull;
+#pragma unroll
+      for (int w = 0; w < NWARP; w++) kmin = min(kmin, (u64)sm.red[w]);
+      if (kmin < best) {
+        if (key == kmin) { sm.tmp = kx; sm.qbase = kw; }  // unique position: one writer
+        __syncthreads();
+        best = kmin;
+        bu = sm.tmp;
+        bw = sm.qbase;
+      }
+      if (best != ~0ull && (int)(best >> 32) == target) break;
+    }
+    __syncthreads();
   }
   // First minimum of psi over Gamma(v) = cadj[s, e) in adjacency order (Alg. 9
   // l.6-11): the G lanes of a group read KB*G consecutive neighbours per step, take
@@ -791,6 +902,43 @@ struct Solver {
   __device__ __forceinline__ int tail_f() const { return p.tail_f > 0 ? p.tail_f : 2 * p.tail_max; }
 
   // ---------------------------------------------------------------- units of work
+  // Single-CTA tail GR levels keep the frontier in shared memory: stage() writes
+  // the next frontier straight into a shared buffer (no flush, no global queue);
+  // entries beyond TQ overflow to the global queue.  After the level: no overflow
+  // -> the frontier stays shared; overflow -> the shared part is appended to the
+  // global queue (the frontier is then global, e.g. for a hand-over to the grid).
+  __device__ void tail_sq_begin(int4 *dst) {
+    sq = true;
+    sq_next = dst;
+    if (threadIdx.x == 0) sm.qcnt = 0;
+    __syncthreads();
+  }
+  // call after the level's barrier; the overflow count is ring_prev(0)
+  __device__ void tail_sq_end(GRState &g, int4 *nxt_global, const int4 *nxt_shared) {
+    sq = false;
+    const int ovf = (int)ring_prev(0), sc = min(sm.qcnt, TQ);
+    if (ovf == 0) {
+      g.nlen = sc;
+      g.in_smem = 1;
+    } else {
+      for (int j = threadIdx.x; j < sc; j += NT) nxt_global[ovf + j] = nxt_shared[j];
+      g.nlen = ovf + sc;
+      g.in_smem = 0;
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) sm.qcnt = 0;
+    __syncthreads();
+  }
+  // a shared frontier must move to the global queue before the grid can see it
+  __device__ void tail_sq_spill(GRState &g) {
+    if (!g.in_smem) return;
+    const int4 *src = sfr(g.cur_is_a ? 0 : 1);
+    int4 *dst = Q4(g.cur_is_a ? 0 : 1);
+    for (int j = threadIdx.x; j < g.nlen; j += NT) dst[j] = src[j];
+    __syncthreads();
+    g.in_smem = 0;
+  }
+
   // GR bookkeeping once the BFS is over (Alg. 7 l.7-9 with GETITERGR, R7)
   __device__ void gr_finish(Ctl &c) {
     int ml = c.gst.deepest + 2;
@@ -805,39 +953,52 @@ struct Solver {
   // GR level 0 (INITRELABEL via the epoch bump + first expansion)
   template <bool GRID>
   __device__ void gr_begin(Ctl &c) {
-    u64 g0 = gtime();
+    u64 g0 = tnow();
     int *U = Ub(c), *T = Tb(c);
-    gr_start<GRID>(c.gst, U, c.ulen, T, Q4(0), c.base, nullptr);
+    if (!GRID && p.tail_ctas == 1) {  // single-CTA tail: the next frontier stays in shared memory
+      tail_sq_begin(sfr(0));  // level 0 fills buffer "a" (gr_start sets cur_is_a = 1)
+      gr_start<GRID>(c.gst, U, c.ulen, T, Q4(0), c.base, nullptr);
+      tail_sq_end(c.gst, Q4(0), sfr(0));
+    } else {
+      gr_start<GRID>(c.gst, U, c.ulen, T, Q4(0), c.base, nullptr);
+      c.gst.in_smem = 0;
+    }
     c.u0 ^= 1;
     c.gr_active = 1;
     if (c.gst.nlen == 0) gr_finish(c);
-    c.ns_gr += (long long)(gtime() - g0);
+    c.ns_gr += (long long)(tnow() - g0);
   }
   // one BFS level (Alg. 5)
   template <bool GRID>
   __device__ void gr_step(Ctl &c) {
-    u64 g0 = gtime();
+    u64 g0 = tnow();
     GRState &g = c.gst;
     g.lvl += 2;
     g.deepest = g.lvl;
-    int4 *cur = Q4(g.cur_is_a ? 0 : 1), *nxt = Q4(g.cur_is_a ? 1 : 0);
+    int4 *cur = g.in_smem ? sfr(g.cur_is_a ? 0 : 1) : Q4(g.cur_is_a ? 0 : 1), *nxt = Q4(g.cur_is_a ? 1 : 0);
     gr_base = c.base;
     trace(2, g.nlen);
+    const bool smemq = !GRID && p.tail_ctas == 1;
+    if (smemq) tail_sq_begin(sfr(g.cur_is_a ? 1 : 0));
     gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
     barrier<GRID>();
-    g.nlen = (int)ring_prev(0);
+    if (smemq) {
+      tail_sq_end(g, nxt, sfr(g.cur_is_a ? 1 : 0));
+    } else {
+      g.nlen = (int)ring_prev(0);
+      g.in_smem = 0;
+    }
     g.cur_is_a ^= 1;
     if (g.nlen == 0) gr_finish(c);
-    c.ns_gr += (long long)(gtime() - g0);
+    c.ns_gr += (long long)(tnow() - g0);
   }
   // one iteration of Alg. 7 l.10-19: fix step (INITKRNL, or SHRKRNL = fix + stable
   // compaction), then PUSHKRNL and the Ac/Ap swap.  Returns false when the fix
   // step found no active column.  The tail group compacts at every step.
   template <bool GRID>
-  __device__ bool loop_step(Ctl &c) {
-    u64 l0 = gtime();
+  __device__ bool loop_step(Ctl &c, int *Ac, int *Ap) {
+    u64 l0 = tnow();
     const u32 cur = c.base - stride();  // epoch of the labels in use
-    int *Ac = Acp(c), *Ap = App(c);
     const int lp = (int)c.loop;
     int act;
     trace(3, c.len);
@@ -863,19 +1024,19 @@ struct Solver {
       // are empty the next fix step compacts, so the tail group can take over
       if (p.compact_adapt && act > 0 && (long long)act * 4 < c.len && c.len > p.tail_max) c.compact_next = 1;
     }
-    debug_check(3, c.loop, Ac, c.len);
+    if (GRID) debug_check(3, c.loop, Ac, c.len);
     if (act == 0) {
-      c.ns_loop += (long long)(gtime() - l0);
+      c.ns_loop += (long long)(tnow() - l0);
       return false;
     }
     trace(4, c.len);
     push<GRID>(c.len, Ac, Ap, lp, cur);
     barrier<GRID>();
-    debug_check(4, c.loop, nullptr, 0);
+    if (GRID) debug_check(4, c.loop, nullptr, 0);
     c.ac0 ^= 1;  // l.18: swap Ac and Ap
     c.loop++;    // l.19
     if (GRID) c.loops++; else c.tail_loops++;
-    c.ns_loop += (long long)(gtime() - l0);
+    c.ns_loop += (long long)(tnow() - l0);
     return true;
   }
 
@@ -892,6 +1053,19 @@ struct Solver {
     Ctrl *x = p.ctrl;
     if (blockIdx.x < p.tail_ctas) {
       const int up = tail_f();
+      bool wl_smem = false;  // the worklist lives in sm.wl (single-CTA tail)
+      auto wl_in = [&]() {
+        if (wl_smem || p.tail_ctas != 1 || c.len > TW) return;
+        for (int i = threadIdx.x; i < c.len; i += NT) { sm.wl[0][i] = __ldcg(p.wl0 + i); sm.wl[1][i] = __ldcg(p.wl1 + i); }
+        __syncthreads();
+        wl_smem = true;
+      };
+      auto wl_out = [&]() {
+        if (!wl_smem) return;
+        for (int i = threadIdx.x; i < c.len; i += NT) { p.wl0[i] = sm.wl[0][i]; p.wl1[i] = sm.wl[1][i]; }
+        __syncthreads();
+        wl_smem = false;
+      };
       for (;;) {
         if (c.loop >= p.max_loops) { reason = R_CAP; break; }
         if (c.gr_active) {
@@ -906,8 +1080,13 @@ struct Solver {
           continue;
         }
         if (c.len > p.tail_max) { reason = R_GRID; break; }
-        if (!loop_step<false>(c)) { reason = R_TERM; break; }
+        wl_in();
+        bool more = wl_smem ? loop_step<false>(c, sm.wl[c.ac0 ? 0 : 1], sm.wl[c.ac0 ? 1 : 0])
+                            : loop_step<false>(c, Acp(c), App(c));
+        if (!more) { reason = R_TERM; break; }
       }
+      wl_out();
+      tail_sq_spill(c.gst);
       if (threadIdx.x == 0 && blockIdx.x == 0) {
         x->ho_reason = reason;
         x->ho_ph = ph;
@@ -916,12 +1095,12 @@ struct Solver {
         for (int j = 0; j < 4; j++) x->ring[j][0] = x->ring[j][1] = x->ring[j][2] = x->ring[j][3] = 0;
       }
     }
+    grid_sync(&p.ctrl->bar, true);
+    nbar++;
     if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
       p.trace[3 * tn] = 99; p.trace[3 * tn + 1] = reason; p.trace[3 * tn + 2] = (long long)gtime();
       tn++;
     }
-    grid_sync(&p.ctrl->bar, true);
-    nbar++;
     reason = (int)ld_rlx((const u32 *)&x->ho_reason);
     ph = (int)ld_rlx((const u32 *)&x->ho_ph) + 1;
     long long *dst = reinterpret_cast<long long *>(&c);
@@ -934,7 +1113,7 @@ struct Solver {
   // maximality (returns false).
   __device__ bool guard_step(Ctl &c) {
     if (!p.final_check) return false;
-    u64 g0 = gtime();
+    u64 g0 = tnow();
     if (base_overflow(c)) { reset_labels(); c.base = 1; }
     int gcount = 0;
     int *Ac = Acp(c), *Ap = App(c);
@@ -944,7 +1123,7 @@ struct Solver {
     c.grs++;
     c.levels += ml / 2;
     c.base += stride();
-    c.ns_gr += (long long)(gtime() - g0);
+    c.ns_gr += (long long)(tnow() - g0);
     if (gcount == 0) return false;
     c.guard_re += gcount;
     for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
@@ -965,12 +1144,12 @@ struct Solver {
   // ---------------------------------------------------------------- the solve
   __device__ void run() {
     const bool lead = blockIdx.x == 0 && threadIdx.x == 0;
-    u64 t0 = gtime(), tA = t0;
+    u64 t0 = tnow(), tA = t0;
     long long ns_init = 0;
     int *Ac = p.wl0, *Ap = p.wl1;
     int *U = p.qa, *T = p.qb;
     int4 *Qa = Q4(0), *Qb = Q4(1);
-    if (threadIdx.x == 0) sm.qcnt = 0;
+    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; }
     init_state();
     barrier<true>();
     if (p.mode == MODE_SOLVE && p.init == 0) {
@@ -1004,7 +1183,7 @@ struct Solver {
 
     barrier<true>();
     debug_check(2, -1, Ac, len);
-    ns_init = (long long)(gtime() - t0);
+    ns_init = (long long)(tnow() - t0);
 
     Ctl c;
     memset(&c, 0, sizeof(c));
@@ -1032,10 +1211,10 @@ struct Solver {
       // one unit of grid work
       if (c.gr_active) { gr_step<true>(c); continue; }                // Alg. 5 level
       if (c.loop == c.gapAt) {                                         // gap relabel (R14)
-        u64 g0 = gtime();
+        u64 g0 = tnow();
         if (gap_relabel(c.base - stride()) >= 0) c.gaps++;
         c.gapAt = -1;
-        c.ns_gr += (long long)(gtime() - g0);
+        c.ns_gr += (long long)(tnow() - g0);
         continue;
       }
       if (c.loop == c.iterGR) {                                        // Alg. 7 l.6-9
@@ -1043,13 +1222,13 @@ struct Solver {
         gr_begin<true>(c);
         continue;
       }
-      if (!loop_step<true>(c) && !guard_step(c)) break;               // l.10-19 / termination
+      if (!loop_step<true>(c, Acp(c), App(c)) && !guard_step(c)) break;  // l.10-19 / termination
     }
     gaps_total = c.gaps;
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
     finish_stats(c.loops + c.tail_loops, c.grs, c.levels, c.shrinks, c.guard_re, init_card, ns_init, c.ns_gr,
-                 c.ns_loop, (long long)(gtime() - tA), c.tail_loops);
+                 c.ns_loop, (long long)(tnow() - tA), c.tail_loops);
   }
 
   __device__ void reset_labels() {

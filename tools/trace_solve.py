@@ -17,6 +17,9 @@ TAGS = {1: "gr_level0", 2: "gr_level", 3: "fix", 4: "push", 0: "other"}
 def summarize(path):
     t = np.fromfile(path, dtype=np.int64).reshape(-1, 3)
     d = np.diff(t[:, 2]) / 1e3  # us; phase i ends at record i+1? record i = end of phase with tag t[i]
+    keep = t[:, 0] < 100  # drop intra-phase marks from the per-phase summary
+    t = t[keep]
+    d = np.diff(t[:, 2]) / 1e3
     tags, sizes = t[1:, 0], t[1:, 1]
     dur = d
     print(f"{len(t)} records, total {(t[-1, 2] - t[0, 2]) / 1e6:.3f} ms")
