@@ -131,24 +131,29 @@ __global__ void k_scan_apply(const int *in, int len, const int *bsum, int *out, 
   if (total_slot >= 0 && b == gridDim.x - 1 && threadIdx.x == 1023) out[total_slot] = ex + x0 + x1;
 }
 
-// scatter rows into Gamma(v) lists: thread per short row, warp per long row
-__global__ void k_scatter(const int *rptr, const int *radj, int m, int *cursor, int *cadj) {
-  int lane = threadIdx.x & 31;
-  long long gw = ((long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-  long long NW = ((long long)gridDim.x * blockDim.x) >> 5;
-  for (long long b = gw * 32; b < m; b += NW * 32) {
-    int u = (int)(b + lane);
-    int s = 0, e = 0;
-    if (u < m) { s = rptr[u]; e = rptr[u + 1]; }
-    if (u < m && e - s <= 32)
-      for (int j = s; j < e; j++) cadj[atomicAdd(cursor + radj[j], 1)] = u;
-    unsigned big = __ballot_sync(0xffffffffu, u < m && e - s > 32);
-    while (big) {
-      int bl = __ffs(big) - 1;
-      big &= big - 1;
-      int ub = __shfl_sync(0xffffffffu, u, bl), sb = __shfl_sync(0xffffffffu, s, bl),
-          eb = __shfl_sync(0xffffffffu, e, bl);
-      for (int j = sb + lane; j < eb; j += 32) cadj[atomicAdd(cursor + radj[j], 1)] = ub;
+// scatter rows into Gamma(v) lists, edge-parallel: warp w owns entries
+// [w*32*SC_K, (w+1)*32*SC_K), lane l the entries base + k*32 + l (coalesced);
+// each lane finds the row of its first entry by binary search in rptr and then
+// walks forward, so a hub row (R-MAT: 1.5e5 entries) is spread over many warps.
+constexpr int SC_K = 8;
+__global__ void k_scatter(const int *rptr, const int *radj, int m, long long nnz, int *cursor, int *cadj) {
+  const int lane = threadIdx.x & 31;
+  const long long warps = ((long long)gridDim.x * blockDim.x) >> 5;
+  for (long long w = ((long long)blockIdx.x * blockDim.x + threadIdx.x) >> 5; w * 32 * SC_K < nnz; w += warps) {
+    const long long base = w * 32 * SC_K;
+    long long e = base + lane;
+    if (e >= nnz) continue;
+    int lo = 0, hi = m - 1;  // largest r with rptr[r] <= e
+    while (lo < hi) {
+      int mid = (lo + hi + 1) >> 1;
+      if (__ldg(rptr + mid) <= e) lo = mid; else hi = mid - 1;
+    }
+    int r = lo, rend = __ldg(rptr + r + 1);
+#pragma unroll 4
+    for (int k = 0; k < SC_K; k++, e += 32) {
+      if (e >= nnz) break;
+      while (e >= rend) rend = __ldg(rptr + (++r) + 1);
+      cadj[atomicAdd(cursor + __ldg(radj + e), 1)] = r;
     }
   }
 }
@@ -292,9 +297,9 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   if (n == 0) CK(cudaMemsetAsync(cptr, 0, sizeof(int), st));
   CK(cudaMemcpyAsync(cursor, cptr, sizeof(int) * ((size_t)n + 1), cudaMemcpyDeviceToDevice, st));
   if (nnz) {
-    int sb = (int)std::min<long long>(((long long)m + 255) / 256, 148 * 16);
-    if (sb < 1) sb = 1;
-    k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, cursor, cadj);
+    long long warps = (nnz + 32 * SC_K - 1) / (32 * SC_K);
+    int sb = (int)std::min<long long>((warps + 7) / 8, 148 * 32);
+    k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, nnz, cursor, cadj);
     CK(cudaGetLastError());
   }
   CK(cudaMemsetAsync(ws + L.hist, 0, sizeof(int) * (size_t)L.hist_len, st));  // zero between gap uses

@@ -299,14 +299,23 @@ struct Solver {
       int s = 0, e = 0;
       if (v < n) { s = ld_ro(p.cptr + v); e = ld_ro(p.cptr + v + 1); }
       if (v < n && e - s <= SMALL_DEG) {
-        for (int j = s; j < e; j++) {
-          int u = ld_ro(p.cadj + j);
-          u64 rs = ld_rlx(p.rowst + u);
-          s_gyedges++;
-          if (mu_of(rs) != -1) continue;
-          if (atomicCAS(p.rowst + u, rs, pack(v, psi_of(rs))) == rs) {
-            st_rlx(p.colst + v, pack(u, 0));
-            break;
+        bool done = false;
+        for (int j0 = s; j0 < e && !done; j0 += KB) {  // KB candidates in flight
+          int u[KB];
+          u64 rs[KB];
+#pragma unroll
+          for (int k = 0; k < KB; k++) u[k] = j0 + k < e ? ld_ro(p.cadj + j0 + k) : -1;
+#pragma unroll
+          for (int k = 0; k < KB; k++) rs[k] = u[k] >= 0 ? ld_rlx(p.rowst + u[k]) : 0ull;
+#pragma unroll
+          for (int k = 0; k < KB; k++) {
+            if (done || u[k] < 0) continue;
+            s_gyedges++;
+            if (mu_of(rs[k]) != -1) continue;
+            if (atomicCAS(p.rowst + u[k], rs[k], pack(v, psi_of(rs[k]))) == rs[k]) {
+              st_rlx(p.colst + v, pack(u[k], 0));
+              done = true;
+            }
           }
         }
       }
