@@ -96,6 +96,9 @@ typedef struct {
                            cluster barrier (the grid then shrinks to whole clusters) */
   int32_t compact_adapt;/* 1 (default): compact the worklist at the next fix step when
                            fewer than 1/4 of its slots hold an active column */
+  int32_t gr_early;     /* 1: a GR stops once every alive unmatched column has a label;
+                           unreached vertices get the next level as a lower bound (R22);
+                           default 1 (ignored when gap = 1); 0 = the paper's complete GR */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 

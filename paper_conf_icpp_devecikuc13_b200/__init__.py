@@ -47,6 +47,7 @@ class Options(ctypes.Structure):
         ("grid_ctas", ctypes.c_int32),
         ("tail_ctas", ctypes.c_int32),
         ("compact_adapt", ctypes.c_int32),
+        ("gr_early", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]
 

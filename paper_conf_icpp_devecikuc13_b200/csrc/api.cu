@@ -202,6 +202,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->tail_f = 128;
   o->tail_ctas = 1;
   o->compact_adapt = 1;
+  o->gr_early = 1;
   o->compact_every = 0;
   o->grid_ctas = 0;
   o->max_loops = 0;
@@ -346,6 +347,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.gap = o.gap; p.final_check = o.final_check; p.dead_skip = o.dead_skip; p.tail_max = o.tail_max;
   p.compact_every = o.compact_every;
   p.compact_adapt = o.compact_adapt;
+  p.gr_early = o.gr_early;
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;

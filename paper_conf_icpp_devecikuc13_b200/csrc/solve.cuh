@@ -49,7 +49,8 @@ struct Ctrl {
   int err;                 // 0 or an MCM_* code
   u32 gcnt;                // exactness-guard list cursor (monotonic within a solve)
   int gmax, gmin;          // gap relabel: largest finite label, smallest empty label
-  int pad[12];
+  u32 ndead;               // columns declared dead (mu = -2), net of guard re-activations
+  int pad[11];
   long long dbg[8];        // debug checks: [0] count, [1] where, [2] loop, [3] vertex, [4] value
   // tail-mode handoff (tail group -> grid): reason, phase counter, Ctl image
   int ho_reason, ho_ph;
@@ -73,7 +74,7 @@ struct Params {
   Ctrl *ctrl;
   // options
   double k;
-  int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt;
+  int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -482,11 +483,16 @@ struct Solver {
         } else {
           s_free++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
+          if (mu_of(cs[k]) != -2) atomicAdd(ring_now(2), 1u);  // an alive unmatched column got its label
         }
       }
     }
   }
   u32 gr_base = 0;
+  int fl_r = 0, fl_c = 0;  // push: labels of vertices the last GR did not reach (set from Ctl)
+  __device__ __forceinline__ int labf(u32 s, u32 base, int stale) const {
+    return s >= base ? (int)min((u64)(s - base), (u64)INF + 1) : stale;
+  }
   bool sq = false;          // tail GR: stage() writes straight into sq_next (shared)
   int4 *sq_next = nullptr;
   __device__ __forceinline__ int4 *sfr(int i) { return reinterpret_cast<int4 *>(sm.q) + i * TQ; }
@@ -507,7 +513,7 @@ struct Solver {
   // The GR as a resumable state machine, so that a CTA-local GR (tail mode) can
   // hand a frontier that grew too wide over to the whole grid mid-BFS.
   struct GRState {
-    int lvl, deepest, nlen, cur_is_a, in_smem, pad;
+    int lvl, deepest, nlen, cur_is_a, in_smem, reached, target, pad;  // reached/target: early stop (R22)
   };
   // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
   template <bool GRID>
@@ -578,6 +584,7 @@ struct Solver {
   // (label, position) minimum per step with the early exit at psi(v)-1 (R11).
   __device__ __forceinline__ void push_finalize(int i, int v, u64 cs, u64 best, int ub, int wb, int loop, u32 base,
                                                 int *Ac, int *Ap) {
+    // (dead columns are counted for the early-stop GR target, R22)
     int psimin = best == ~0ull ? INF : (int)(best >> 32);
     if (psimin < INF) {                                 // l.12
       if (wb == -1 || ld_rlx(p.iA + wb) != loop) {      // l.13
@@ -594,6 +601,7 @@ struct Solver {
       Ac[i] = -1;                                       // l.21
       Ap[i] = -1;                                       // l.22
       s_dead++;
+      atomicAdd(&p.ctrl->ndead, 1u);
     }
   }
 
@@ -610,7 +618,7 @@ struct Solver {
       u64 cs = 0;
       if (v >= 0) {
         cs = ld_rlx(p.colst + v);
-        psiv = lab(psi_of(cs), base, INF);
+        psiv = labf(psi_of(cs), base, fl_c);
         s = ld_ro(p.cptr + v);
         e = ld_ro(p.cptr + v + 1);
         if (p.dead_skip && psiv >= INF) e = s;  // R19: provably unmatchable
@@ -688,7 +696,7 @@ struct Solver {
       for (int k = 0; k < KB; k++) {
         if (x[k] < 0) continue;
         s_scan++;
-        int l = lab(psi_of(rs[k]), base, INF);
+        int l = labf(psi_of(rs[k]), base, fl_r);
         u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + (int)threadIdx.x + k * NT - s)) : ~0ull;
         if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
       }
@@ -740,7 +748,7 @@ struct Solver {
       for (int k = 0; k < KB; k++) {
         if (x[k] < 0) continue;
         s_scan++;
-        int l = lab(psi_of(rs[k]), base, INF);
+        int l = labf(psi_of(rs[k]), base, fl_r);
         u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + gl + k * G - s)) : ~0ull;
         if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
       }
@@ -886,6 +894,7 @@ struct Solver {
     int len, ulen;
     u32 base;
     int shrink, compact_next, gr_active, ac0, u0, pad;
+    int floor_r, floor_c;  // labels of vertices the last GR did not reach (m+n unless it stopped early)
     GRState gst;
     // statistics (meaningful in the lead thread)
     long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop;
@@ -908,6 +917,7 @@ struct Solver {
   }
   // GR frontiers of at most tail_f() rows run on the tail group (hand-over back to
   // the grid when a frontier outgrows it, back to the tail below tail_f()/2)
+  __device__ __forceinline__ bool early_gr() const { return p.gr_early && !p.gap; }
   __device__ __forceinline__ int tail_f() const { return p.tail_f > 0 ? p.tail_f : 2 * p.tail_max; }
 
   // ---------------------------------------------------------------- units of work
@@ -949,7 +959,13 @@ struct Solver {
   }
 
   // GR bookkeeping once the BFS is over (Alg. 7 l.7-9 with GETITERGR, R7)
-  __device__ void gr_finish(Ctl &c) {
+  __device__ void gr_finish(Ctl &c, bool early = false) {
+    // complete BFS: unreached = infinite (Alg. 2); early stop (R22) after expanding
+    // the rows of level l: unreached columns >= l+3, rows >= l+4 (lower bounds that
+    // keep the neighbourhood invariant next to the unexpanded rows of level l+2)
+    c.floor_c = early ? c.gst.lvl + 3 : INF;
+    c.floor_r = early ? c.gst.lvl + 4 : INF;
+    if (early) c.gst.deepest = c.gst.lvl + 2;
     int ml = c.gst.deepest + 2;
     c.grs++;
     c.levels += ml / 2;
@@ -974,7 +990,12 @@ struct Solver {
     }
     c.u0 ^= 1;
     c.gr_active = 1;
+    // early stop (R22): every alive unmatched column is active; stop once all of them
+    // carry a label.  alive unmatched = n - matched - dead; matched = m - |U|.
+    c.gst.reached = (int)ring_prev(2);
+    c.gst.target = early_gr() ? n - (m - c.ulen) - (int)ld_rlx((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
     if (c.gst.nlen == 0) gr_finish(c);
+    else if (c.gst.reached >= c.gst.target) gr_finish(c, true);
     c.ns_gr += (long long)(tnow() - g0);
   }
   // one BFS level (Alg. 5)
@@ -998,7 +1019,9 @@ struct Solver {
       g.in_smem = 0;
     }
     g.cur_is_a ^= 1;
+    g.reached += (int)ring_prev(2);
     if (g.nlen == 0) gr_finish(c);
+    else if (g.reached >= g.target) gr_finish(c, true);
     c.ns_gr += (long long)(tnow() - g0);
   }
   // one iteration of Alg. 7 l.10-19: fix step (INITKRNL, or SHRKRNL = fix + stable
@@ -1039,6 +1062,8 @@ struct Solver {
       return false;
     }
     trace(4, c.len);
+    fl_r = c.floor_r;
+    fl_c = c.floor_c;
     push<GRID>(c.len, Ac, Ap, lp, cur);
     barrier<GRID>();
     if (GRID) debug_check(4, c.loop, nullptr, 0);
@@ -1138,12 +1163,14 @@ struct Solver {
     for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
       int v = __ldcg(Ac + i);
       u64 cs = ld_rlx(p.colst + v);
+      if (mu_of(cs) == -2) atomicSub(&p.ctrl->ndead, 1u);
       st_rlx(p.colst + v, pack(-1, psi_of(cs)));
       Ap[i] = v;
     }
     barrier<true>();
     if (blockIdx.x == 0 && threadIdx.x == 0) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
     c.len = gcount;
+    c.floor_r = c.floor_c = INF;
     c.iterGR = c.loop + iter_gap(ml);
     c.gapAt = gap_at(c.loop, c.iterGR);
     c.shrink = 0;
@@ -1197,6 +1224,7 @@ struct Solver {
     Ctl c;
     memset(&c, 0, sizeof(c));
     c.len = len; c.ulen = ulen; c.base = 1; c.gapAt = -1; c.ac0 = 1; c.u0 = 1;  // loop = iterGR = 0
+    c.floor_r = c.floor_c = INF;
     for (;;) {
       if (c.loop >= p.max_loops) {
         if (lead) p.ctrl->err = -5;
