@@ -99,6 +99,12 @@ typedef struct {
   int32_t gr_early;     /* 1: a GR stops once every alive unmatched column has a label;
                            unreached vertices get the next level as a lower bound (R22);
                            default 1 (ignored when gap = 1); 0 = the paper's complete GR */
+  int32_t serial;       /* 1 (tests): the fix and push steps run on one thread with the slots
+                           in increasing order, GRs complete, no tail / adaptive compaction:
+                           the trajectory of the serial simulator (oracle or_gpr_serial);
+                           default 0 */
+  int32_t sort_csc;     /* mcm_create: 1 = sort every Gamma(v) by row id (deterministic scan
+                           order, needed for bit-exact serial runs); default 0 */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 

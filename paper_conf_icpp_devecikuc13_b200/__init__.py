@@ -48,6 +48,8 @@ class Options(ctypes.Structure):
         ("tail_ctas", ctypes.c_int32),
         ("compact_adapt", ctypes.c_int32),
         ("gr_early", ctypes.c_int32),
+        ("serial", ctypes.c_int32),
+        ("sort_csc", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]
 

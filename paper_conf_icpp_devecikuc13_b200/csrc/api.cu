@@ -136,6 +136,17 @@ __global__ void k_scan_apply(const int *in, int len, const int *bsum, int *out, 
 // each lane finds the row of its first entry by binary search in rptr and then
 // walks forward, so a hub row (R-MAT: 1.5e5 entries) is spread over many warps.
 constexpr int SC_K = 8;
+// optional: sort every Gamma(v) by row id (insertion sort, thread per column; tests)
+__global__ void k_sort_segments(const int *cptr, int *cadj, int n) {
+  for (long long v = (long long)blockIdx.x * blockDim.x + threadIdx.x; v < n; v += (long long)gridDim.x * blockDim.x) {
+    int s = cptr[v], e = cptr[v + 1];
+    for (int i = s + 1; i < e; i++) {
+      int x = cadj[i], j = i - 1;
+      while (j >= s && cadj[j] > x) { cadj[j + 1] = cadj[j]; j--; }
+      cadj[j + 1] = x;
+    }
+  }
+}
 __global__ void k_scatter(const int *rptr, const int *radj, int m, long long nnz, int *cursor, int *cadj) {
   const int lane = threadIdx.x & 31;
   const long long warps = ((long long)gridDim.x * blockDim.x) >> 5;
@@ -302,6 +313,10 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
     int sb = (int)std::min<long long>((warps + 7) / 8, 148 * 32);
     k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, nnz, cursor, cadj);
     CK(cudaGetLastError());
+    if (h->opt.sort_csc) {
+      k_sort_segments<<<(n + 255) / 256, 256, 0, st>>>(cptr, cadj, n);
+      CK(cudaGetLastError());
+    }
   }
   CK(cudaMemsetAsync(ws + L.hist, 0, sizeof(int) * (size_t)L.hist_len, st));  // zero between gap uses
   CK(cudaStreamSynchronize(st));
@@ -348,6 +363,13 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.compact_every = o.compact_every;
   p.compact_adapt = o.compact_adapt;
   p.gr_early = o.gr_early;
+  p.serial = o.serial;
+  if (o.serial) {  // the simulator's schedule: complete GRs, no tail, no adaptive compaction
+    p.tail_max = 0;
+    p.gr_early = 0;
+    p.compact_adapt = 0;
+    p.compact_every = 0;
+  }
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;

@@ -75,6 +75,7 @@ struct Params {
   // options
   double k;
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
+  int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -1142,6 +1143,83 @@ struct Solver {
     return reason;
   }
 
+  // Serial mode (tests): one thread runs the fix and push steps of Alg. 7 with the
+  // slots in increasing order -- exactly the schedule of the oracle's serial
+  // simulator (oracle.c or_gpr_serial) -- until a GR (which runs on the grid, as
+  // always) or a gap relabel is due, or no active column is left.  Trajectory,
+  // matching and counters are then bit-exact against the simulator.
+  __device__ void serial_fix_push(Ctl &c, int &reason) {
+    const u32 base = c.base - stride();
+    for (;;) {
+      if (c.loop >= p.max_loops) { reason = R_CAP; return; }
+      if (c.loop == c.gapAt || c.loop == c.iterGR) { reason = R_GRID; return; }
+      int *Ac = Acp(c), *Ap = App(c);
+      const int loop = (int)c.loop;
+      bool act = false;
+      s_slots += c.len;
+      if (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) {  // SHRKRNL, slot order
+        int out = 0;
+        for (int i = 0; i < c.len; i++) {
+          int v = Ap[i], a = Ac[i];
+          if (v != -1 && col_unmatched(v)) a = v;
+          if (a != -1) { st_rlx(p.iA + a, loop); act = true; Ac[out++] = a; }
+        }
+        c.len = out;
+        c.shrinks++;
+        c.shrink = 0;
+      } else {  // INITKRNL (Alg. 8)
+        for (int i = 0; i < c.len; i++) {
+          int v = Ap[i];
+          if (v != -1 && col_unmatched(v)) Ac[i] = v;
+          v = Ac[i];
+          if (v != -1) { st_rlx(p.iA + v, loop); act = true; }
+        }
+      }
+      if (!act) { reason = R_TERM; return; }
+      for (int i = 0; i < c.len; i++) {  // PUSHKRNL (Alg. 9)
+        int v = Ac[i];
+        if (v == -1) { Ap[i] = -1; continue; }
+        u64 cs = ld_rlx(p.colst + v);
+        int psiv = labf(psi_of(cs), base, INF);
+        int s = ld_ro(p.cptr + v), e = ld_ro(p.cptr + v + 1);
+        if (p.dead_skip && psiv >= INF) e = s;
+        int psimin = INF, ub = -1, wb = -1;
+        for (int j = s; j < e; j++) {
+          int x = ld_ro(p.cadj + j);
+          u64 rs = ld_rlx(p.rowst + x);
+          int l = labf(psi_of(rs), base, INF);
+          s_scan++;
+          if (l < psimin) {
+            psimin = l; ub = x; wb = mu_of(rs);
+            if (psimin == psiv - 1) break;
+          }
+        }
+        u64 best = psimin < INF ? ((u64)(u32)psimin << 32) : ~0ull;
+        push_finalize(i, v, cs, best, ub, wb, loop, base, Ac, Ap);
+      }
+      c.ac0 ^= 1;
+      c.loop++;
+      c.loops++;
+    }
+  }
+  __device__ int serial_episode(Ctl &c) {
+    int reason = R_NONE;
+    Ctrl *x = p.ctrl;
+    if (threadIdx.x == 0 && blockIdx.x == 0) {
+      serial_fix_push(c, reason);
+      x->ho_reason = reason;
+      x->ho_ph = ph;
+      const long long *src = reinterpret_cast<const long long *>(&c);
+      for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) x->ho[j] = src[j];
+    }
+    grid_sync(&p.ctrl->bar, false);
+    nbar++;
+    reason = (int)ld_rlx((const u32 *)&x->ho_reason);
+    long long *dst = reinterpret_cast<long long *>(&c);
+    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) dst[j] = ld_rlx(&x->ho[j]);
+    return reason;
+  }
+
   // exactness guard (R16): one more GR; every unmatched column it reaches is
   // re-activated and the loop resumes (returns true); otherwise the labels certify
   // maximality (returns false).
@@ -1229,6 +1307,15 @@ struct Solver {
       if (c.loop >= p.max_loops) {
         if (lead) p.ctrl->err = -5;
         break;
+      }
+      if (p.serial && !c.gr_active && c.loop != c.iterGR && c.loop != c.gapAt) {
+        int r = serial_episode(c);
+        if (r == R_CAP) {
+          if (lead) p.ctrl->err = -5;
+          break;
+        }
+        if (r == R_TERM && !guard_step(c)) break;
+        continue;
       }
       const int up = tail_f();
       bool tail_ok = p.tail_max > 0 &&

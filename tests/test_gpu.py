@@ -251,3 +251,46 @@ def test_gap_solves_exact_without_guard():
         card, st = check_solve(g, gap=1, final_check=0)
         card2, st2 = check_solve(g, gap=1, final_check=1)
         assert st2["guard_reactivated"] == 0
+
+
+# ---------------------------------------------------------------- serial mode, bit-exact trajectory
+SERIAL_CASES = [
+    (lambda: synth.config("C1", 0.3), {}), (lambda: synth.config("C2", 0.003), {}),
+    (lambda: synth.config("C3", 0.0005), {}), (lambda: synth.config("C4", 1 / 2048), {}),
+    (lambda: synth.hall_violator(800, 60, 17, 3), {}), (lambda: synth.complete(30, 20), {}),
+    (lambda: synth.config("C1", 0.3), dict(k=2.0)), (lambda: synth.config("C1", 0.3), dict(gr_fixed=True, k=10)),
+    (lambda: synth.config("C2", 0.003), dict(shrink_min=-1)), (lambda: synth.config("C4", 1 / 2048), dict(dead_skip=True)),
+    (lambda: synth.config("C1", 0.3), dict(gap=True)), (lambda: synth.config("C4", 1 / 2048), dict(gap=True)),
+]
+
+
+@pytest.mark.parametrize("ci", range(len(SERIAL_CASES)))
+def test_serial_mode_matches_simulator(ci):
+    """With the slots processed in order by one thread (options serial=1, sorted
+    CSC), the GPU run reproduces the oracle's serial simulator of Alg. 7/8/9
+    (or_gpr_serial) exactly: final mu arrays, cardinality, loop / GR / push /
+    dead / blocked / shrink counts.  Pins the fix, shrink, push, iA-guard,
+    rollback, GR and GETITERGR logic of the CUDA path, not just its result."""
+    mk, kw = SERIAL_CASES[ci]
+    g = mk()
+    csc = oracle.transpose(g)
+    _, rm0, cm0 = oracle.cheap_match(g, csc)
+    sim_kw = dict(k=kw.get("k", 0.7), gr_fixed=kw.get("gr_fixed", False), shrink_min=kw.get("shrink_min", 512),
+                  dead_skip=kw.get("dead_skip", False), gap=kw.get("gap", False))
+    card, srm, scm, st = oracle.gpr_serial(g, init=(rm0, cm0), csc=csc, **sim_kw)
+    opts = dict(serial=1, sort_csc=1, init="given", final_check=0, k=sim_kw["k"],
+                gr_strategy="fixed" if sim_kw["gr_fixed"] else "adaptive", shrink_min=sim_kw["shrink_min"],
+                dead_skip=int(sim_kw["dead_skip"]), gap=int(sim_kw["gap"]))
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, **opts)
+    rm = torch.from_numpy(rm0.astype(np.int32)).to(DEV)
+    cm = torch.from_numpy(cm0.astype(np.int32)).to(DEV)
+    gcard, grm, gcm = mt.solve(rm, cm)
+    gst = mt.stats()
+    mt.close()
+    assert gcard == card
+    assert np.array_equal(grm.cpu().numpy(), srm) and np.array_equal(gcm.cpu().numpy(), scm), g.name
+    got = dict(loops=gst["loops"], grs=gst["gr_count"], levels=gst["gr_levels"], pushes=gst["pushes"],
+               shrinks=gst["shrinks"], dead=gst["dead"], blocked=gst["blocked"], gaps=gst["gaps"])
+    want = {k: st[k] for k in got}
+    assert got == want, (g.name, kw, got, want)
