@@ -105,6 +105,9 @@ typedef struct {
                            default 0 */
   int32_t sort_csc;     /* mcm_create: 1 = sort every Gamma(v) by row id (deterministic scan
                            order, needed for bit-exact serial runs); default 0 */
+  int32_t variant;      /* 0 (default): G-PR (Alg. 7, active-column worklist);
+                           1: G-PR-First (Alg. 3 + Alg. 6: every column
+                           tested every loop; the Fig. 1 ablation) */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 

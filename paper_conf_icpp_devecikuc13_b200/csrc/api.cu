@@ -249,6 +249,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
     return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
+  if (o->variant < 0 || o->variant > 1) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -364,6 +365,11 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.compact_adapt = o.compact_adapt;
   p.gr_early = o.gr_early;
   p.serial = o.serial;
+  p.variant = o.variant;
+  if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either
+    p.tail_max = 0;
+    p.serial = 0;
+  }
   if (o.serial) {  // the simulator's schedule: complete GRs, no tail, no adaptive compaction
     p.tail_max = 0;
     p.gr_early = 0;

@@ -76,6 +76,7 @@ struct Params {
   double k;
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
+  int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -1220,6 +1221,50 @@ struct Solver {
     return reason;
   }
 
+  // G-PR-First (Alg. 3 + Alg. 6; the Fig. 1 ablation,
+  // SURVEY NEXT-1): every loop tests every column for activity (R1) and pushes the
+  // active ones -- no worklist, no iA.  One thread per column, batched scan.
+  __device__ bool first_step(Ctl &c) {
+    u64 l0 = tnow();
+    const u32 base = c.base - stride();
+    const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    long long act = 0;
+    fl_r = c.floor_r;
+    fl_c = c.floor_c;
+    for (int v = g; v < n; v += G) {
+      u64 cs = ld_rlx(p.colst + v);
+      int cm = mu_of(cs);
+      bool active = cm == -1 || (cm >= 0 && mu_of(ld_rlx(p.rowst + cm)) != v);  // Alg. 6 l.3 (R1)
+      if (!active) continue;
+      act++;
+      int psiv = labf(psi_of(cs), base, fl_c);
+      int s = ld_ro(p.cptr + v), e = ld_ro(p.cptr + v + 1);
+      if (p.dead_skip && psiv >= INF) e = s;
+      u64 best;
+      int ub, wb;
+      scan(s, e, 0, 1, 1u << lane_id(), psiv - 1, base, best, ub, wb);  // l.5-12
+      int psimin = best == ~0ull ? INF : (int)(best >> 32);
+      if (psimin < INF) {                                             // l.13-17
+        st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));
+        st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));
+        s_push++;
+      } else {                                                        // l.18-19
+        st_rlx(p.colst + v, pack(-2, psi_of(cs)));
+        s_dead++;
+        atomicAdd(&p.ctrl->ndead, 1u);
+      }
+    }
+    trace(4, n);
+    add_count(act, 0);
+    barrier<true>();
+    const long long a = ring_prev(0);
+    c.ns_loop += (long long)(tnow() - l0);
+    if (a == 0) return false;
+    c.loop++;
+    c.loops++;
+    return true;
+  }
+
   // exactness guard (R16): one more GR; every unmatched column it reaches is
   // re-activated and the loop resumes (returns true); otherwise the labels certify
   // maximality (returns false).
@@ -1344,6 +1389,10 @@ struct Solver {
       if (c.loop == c.iterGR) {                                        // Alg. 7 l.6-9
         if (base_overflow(c)) { reset_labels(); c.base = 1; }
         gr_begin<true>(c);
+        continue;
+      }
+      if (p.variant == 1) {                                             // G-PR-First (Alg. 3)
+        if (!first_step(c) && !guard_step(c)) break;
         continue;
       }
       if (!loop_step<true>(c, Acp(c), App(c)) && !guard_step(c)) break;  // l.10-19 / termination
