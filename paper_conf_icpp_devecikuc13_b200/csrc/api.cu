@@ -24,7 +24,7 @@ constexpr int MAX_CTAS = 4096;
 size_t align256(size_t x) { return (x + 255) & ~(size_t)255; }
 
 struct Layout {
-  size_t ctrl, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, dbg, total;
+  size_t ctrl, ovf, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, dbg, total;
   int hist_len;
 };
 
@@ -34,6 +34,7 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   auto take = [&](size_t bytes) { size_t r = o; o += align256(bytes > 0 ? bytes : 1); return r; };
   size_t mx = (size_t)(m > n ? m : n) + 1;
   L.ctrl = take(sizeof(Ctrl));
+  L.ovf = take(sizeof(int4) * mx);
   L.rptr = take(sizeof(int) * ((size_t)m + 1));
   L.radj = take(sizeof(int) * (size_t)nnz);
   L.cptr = take(sizeof(int) * ((size_t)n + 1));
@@ -214,6 +215,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->tail_ctas = 1;
   o->compact_adapt = 1;
   o->gr_early = 1;
+  o->bu_div = 16;
   o->compact_every = 0;
   o->grid_ctas = 0;
   o->max_loops = 0;
@@ -249,7 +251,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
     return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
-  if (o->variant < 0 || o->variant > 1) return MCM_EINVAL;
+  if (o->variant < 0 || o->variant > 1 || o->bu_div < 0) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -347,6 +349,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.ctrl = (Ctrl *)(ws + L.ctrl);
   p.dbgbuf = (int *)(ws + L.dbg);
   p.hist = (int *)(ws + L.hist);
+  p.ovf = (int4 *)(ws + L.ovf);
+  p.ovf_len = (long long)((h->m > h->n ? h->m : h->n) + 1);
   p.hist_len = L.hist_len;
   p.debug = getenv("MCM_DEBUG") ? atoi(getenv("MCM_DEBUG")) : 0;
   // MCM_TRACE=<n>: record up to n phase boundaries into the (otherwise idle during
@@ -366,6 +370,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.gr_early = o.gr_early;
   p.serial = o.serial;
   p.variant = o.variant;
+  p.bu_div = o.bu_div;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either
     p.tail_max = 0;
     p.serial = 0;

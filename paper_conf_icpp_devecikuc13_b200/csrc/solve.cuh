@@ -42,7 +42,7 @@ enum {
 };
 
 struct Ctrl {
-  u32 ring[4][4];          // per-phase counters, rotated (see Solver::barrier)
+  u32 ring[4][8];          // per-phase counters, rotated (see Solver::barrier)
   u32 bar;                 // grid barrier word (device.cuh grid_sync)
   u32 pad0[3];
   long long stat[ST_NSTAT];
@@ -67,6 +67,8 @@ struct Params {
   int tail_ctas;           // CTAs of the tail group (= cluster 0 when > 1)
   int tail_f;              // GR frontier limit of the tail group (0: 2 * tail_max)
   int *hist;               // gap relabel histogram (hist_len counters, zero between uses)
+  int4 *ovf;               // per-CTA overflow regions of the BFS frontier staging
+  long long ovf_len;       // entries in ovf
   int hist_len;
   int debug;
   long long *trace;        // optional phase trace: {tag, size, t_end_ns} triples (MCM_TRACE)
@@ -77,12 +79,15 @@ struct Params {
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
+  int bu_div;              // bottom-up BFS level when frontier * bu_div >= n (0: top-down only)
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
   int *rmatch_out, *cmatch_out;  // solve: matching; relabel: psi_row / psi_col
 };
 
+struct Smem;
+extern __shared__ Smem smem_dyn[];
 struct Smem {
   long long red[NWARP];
   int w[NWARP];
@@ -109,7 +114,10 @@ __device__ __forceinline__ u64 tnow() { return (threadIdx.x == 0 && blockIdx.x =
 
 struct Solver {
   const Params &p;
-  Smem &sm;
+  // the dynamic shared block, named through a namespace-scope extern __shared__
+  // array so every access compiles to a shared-space instruction (a Smem& member
+  // made the staging atomics generic ATOM.E)
+#define sm (smem_dyn[0])
   const int m, n, INF;
   // per-thread statistics (reduced at the end)
   long long s_push = 0, s_block = 0, s_dead = 0, s_scan = 0, s_slots = 0, s_free = 0;
@@ -129,7 +137,11 @@ struct Solver {
     }
   }
 
-  __device__ Solver(const Params &p_, Smem &sm_) : p(p_), sm(sm_), m(p_.m), n(p_.n), INF(p_.m + p_.n) {}
+  int ovf_r = 0;  // entries of this CTA's overflow region
+  int n_iso = 0;  // rows without edges (excluded from U in solve mode)
+  __device__ Solver(const Params &p_) : p(p_), m(p_.m), n(p_.n), INF(p_.m + p_.n) {
+    ovf_r = (int)(p_.ovf_len / gridDim.x);
+  }
 
   // ---------------------------------------------------------------- barriers
   // ring[ph & 3] collects the counts produced during phase ph; the consumer reads
@@ -156,7 +168,8 @@ struct Solver {
     ph++;
     if (blockIdx.x == 0 && threadIdx.x == 0) {
       u32 *r = p.ctrl->ring[(ph + 2) & 3];
-      r[0] = r[1] = r[2] = r[3] = 0;
+#pragma unroll
+      for (int j = 0; j < 8; j++) r[j] = 0;
     }
   }
   __device__ __forceinline__ u32 *ring_now(int j) { return &p.ctrl->ring[ph & 3][j]; }
@@ -194,7 +207,9 @@ struct Solver {
     int q = base + (int)g.thread_rank();
     if (q < (sq ? TQ : QCAP4)) {
       (sq ? sq_next : reinterpret_cast<int4 *>(sm.q))[q] = x;
-    } else {  // overflow: direct append, again one global atomic per group
+    } else if (!sq && q - QCAP4 < ovf_r) {  // overflow: this CTA's private global region
+      p.ovf[(long long)blockIdx.x * ovf_r + (q - QCAP4)] = x;
+    } else {  // region full too: direct append, one global atomic per group
       cg::coalesced_group o = cg::coalesced_threads();
       u32 gb = 0;
       if (o.thread_rank() == 0) gb = atomicAdd(gcnt, (u32)o.size());
@@ -205,10 +220,24 @@ struct Solver {
   __device__ __forceinline__ void flush(int4 *next, u32 *gcnt) {
     if (sq) return;  // tail: the next frontier is the shared buffer itself
     __syncthreads();
-    int c = min(sm.qcnt, QCAP4);
-    if (threadIdx.x == 0) sm.qbase = c ? (int)atomicAdd(gcnt, (u32)c) : 0;
+    // one reservation per CTA and tile for the shared entries and the private
+    // overflow region (wide levels would otherwise serialise on one counter)
+    const int c = min(sm.qcnt, QCAP4), co = min(max(sm.qcnt - QCAP4, 0), ovf_r);
+    if (threadIdx.x == 0) sm.qbase = (c + co) ? (int)atomicAdd(gcnt, (u32)(c + co)) : 0;
     __syncthreads();
-    for (int j = threadIdx.x; j < c; j += NT) next[sm.qbase + j] = reinterpret_cast<const int4 *>(sm.q)[j];
+    u32 fe = 0;  // adjacency entries of the next frontier (direction choice)
+    for (int j = threadIdx.x; j < c; j += NT) {
+      const int4 q = reinterpret_cast<const int4 *>(sm.q)[j];
+      next[sm.qbase + j] = q;
+      fe += (u32)(q.z - q.y);
+    }
+    for (int j = threadIdx.x; j < co; j += NT) {
+      const int4 q = __ldcg(p.ovf + (long long)blockIdx.x * ovf_r + j);
+      next[sm.qbase + c + j] = q;
+      fe += (u32)(q.z - q.y);
+    }
+    fe = __reduce_add_sync(0xffffffffu, fe);
+    if (lane_id() == 0 && fe) atomicAdd(ring_now(4), fe);
     __syncthreads();
     if (threadIdx.x == 0) sm.qcnt = 0;
     __syncthreads();
@@ -351,15 +380,20 @@ struct Solver {
   }
 
   // unmatched rows -> U (any order); ring j
+  // solve mode: rows without any edge can never be matched nor reach a column, so
+  // they stay out of U (their count goes to ring counter j+1)
   __device__ void build_unmatched_rows(int *U, int j) {
+    long long iso = 0;
     for (int t = blockIdx.x * NT; t < m; t += gridDim.x * NT) {
       int u = t + threadIdx.x;
       bool f = u < m && mu_of(ld_rlx(p.rowst + u)) == -1;
+      if (f && p.mode == MODE_SOLVE && ld_ro(p.rptr + u) == ld_ro(p.rptr + u + 1)) { f = false; iso++; }
       int tot, r = cta_rank<NT>(f, sm.w, &tot);
       if (threadIdx.x == 0) sm.qbase = tot ? (int)atomicAdd(ring_now(j), (u32)tot) : 0;
       __syncthreads();
       if (f) U[sm.qbase + r] = u;
     }
+    add_count(iso, j + 1);
   }
 
   // ---------------------------------------------------------------- global relabel
@@ -478,6 +512,7 @@ struct Solver {
       for (int k = 0; k < KB; k++) {
         if (old[k] != cs[k]) continue;  // not claimed by this thread
         s_grcols++;
+        lvl_cols++;
         int w = mu_of(cs[k]);
         if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: mu(v) > -1 and mu(mu(v)) = v
           st_rlx(p.rowst + w, pack(v[k], lr));
@@ -490,7 +525,96 @@ struct Solver {
       }
     }
   }
+  // Bottom-up BFS level (direction-optimising GR): every column
+  // not yet labelled in this GR looks for any row of Gamma(v) carrying the
+  // current level `lvl`, stopping at the first one; a hit labels v lvl+1 and, if v
+  // is matched, its mate lvl+2 (staged for the next level).  Produces exactly the
+  // labels of the top-down level (BFS distances are unique) while reading a
+  // fraction of the adjacency on wide levels.  One thread per column (no CAS:
+  // each column is visited by its own thread); lists longer than BIG_DEG are
+  // scanned by the whole warp with the same early exit.
+  template <bool GRID>
+  __device__ void gr_level_bu(int lvl, u32 base, int4 *next, u32 *ncnt, int *guard, u32 *gcnt) {
+    const int lane = lane_id();
+    const u32 lf = base + lvl, lc = base + lvl + 1, lr = base + lvl + 2;
+    for (int t = cta<GRID>() * NT; t < n; t += ncta<GRID>() * NT) {
+      const int v = t + (int)threadIdx.x;
+      u64 cs = 0;
+      int s = 0, e = 0;
+      bool open = false, hit = false;
+      if (v < n) {
+        cs = ld_rlx(p.colst + v);
+        if (psi_of(cs) < base) {
+          open = true;
+          s = ld_ro(p.cptr + v);
+          e = ld_ro(p.cptr + v + 1);
+        }
+      }
+      if (open && e - s <= BIG_DEG) {
+        for (int j = s; j < e && !hit; j += KB) {
+          int x[KB];
+          u64 rs[KB];
+#pragma unroll
+          for (int k = 0; k < KB; k++) x[k] = j + k < e ? ld_ro(p.cadj + j + k) : -1;
+#pragma unroll
+          for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+#pragma unroll
+          for (int k = 0; k < KB; k++) hit |= x[k] >= 0 && psi_of(rs[k]) == lf;
+          s_gredges += min(KB, e - j);
+        }
+      }
+      unsigned bigm = __ballot_sync(0xffffffffu, open && e - s > BIG_DEG);
+      while (bigm) {  // long lists: the whole warp, exit at the first hit
+        const int bl = __ffs(bigm) - 1;
+        bigm &= bigm - 1;
+        const int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
+        bool any = false;
+        for (int c0 = sb; c0 < eb && !any; c0 += 32 * KB) {
+          bool h = false;
+#pragma unroll
+          for (int k = 0; k < KB; k++) {
+            const int jj = c0 + k * 32 + lane;
+            if (jj < eb) h |= psi_of(ld_rlx(p.rowst + ld_ro(p.cadj + jj))) == lf;
+          }
+          any = __any_sync(0xffffffffu, h);
+          if (lane == 0) s_gredges += min(32 * KB, eb - c0);
+        }
+        if (lane == bl) hit = any;
+      }
+      if (hit) {
+        st_rlx(p.colst + v, pack(mu_of(cs), lc));
+        s_grcols++;
+        lvl_cols++;
+        const int w = mu_of(cs);
+        u64 rw = 0;
+        int rs = 0, re = 0;
+        if (w >= 0) { rw = ld_rlx(p.rowst + w); rs = ld_ro(p.rptr + w); re = ld_ro(p.rptr + w + 1); }
+        if (w >= 0 && mu_of(rw) == v) {  // matched: its mate joins the next level
+          st_rlx(p.rowst + w, pack(v, lr));
+          stage(make_int4(w, rs, re, 0), next, ncnt);
+        } else {
+          s_free++;
+          if (guard) guard[atomicAdd(gcnt, 1u)] = v;
+          if (w != -2) atomicAdd(ring_now(2), 1u);
+        }
+      }
+      flush(next, ncnt);
+    }
+  }
+  // bottom-up when the frontier's adjacency entries reach bu_div/8 times the
+  // columns still unlabelled (Beamer-style edge rule; frontier rows alone mislead on
+  // low-degree road graphs)
+  __device__ __forceinline__ bool use_bottom_up(long long fedges, long long unvisited) const {
+    return p.bu_div > 0 && fedges * 8 >= unvisited * (long long)p.bu_div;
+  }
+
   u32 gr_base = 0;
+  u32 lvl_cols = 0;  // columns this thread labelled in the current level
+  __device__ __forceinline__ void level_cols_flush() {
+    u32 x = __reduce_add_sync(0xffffffffu, lvl_cols);
+    if (lane_id() == 0 && x) atomicAdd(ring_now(5), x);
+    lvl_cols = 0;
+  }
   int fl_r = 0, fl_c = 0;  // push: labels of vertices the last GR did not reach (set from Ctl)
   __device__ __forceinline__ int labf(u32 s, u32 base, int stale) const {
     return s >= base ? (int)min((u64)(s - base), (u64)INF + 1) : stale;
@@ -516,6 +640,7 @@ struct Solver {
   // hand a frontier that grew too wide over to the whole grid mid-BFS.
   struct GRState {
     int lvl, deepest, nlen, cur_is_a, in_smem, reached, target, pad;  // reached/target: early stop (R22)
+    long long fedges, visited;  // next frontier's adjacency entries; columns labelled in this GR
   };
   // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
   template <bool GRID>
@@ -524,8 +649,11 @@ struct Solver {
     u32 *gc = &p.ctrl->gcnt;  // zero here: reset one phase after its last use
     trace(1, ulen);
     gr_level<GRID>(U, nullptr, ulen, 0, base, Qa, ring_now(0), T, ring_now(1), guard, gc);
+    level_cols_flush();
     barrier<GRID>();
     g.nlen = (int)ring_prev(0);
+    g.fedges = ring_prev(4);
+    g.visited = ring_prev(5);
     ulen = (int)ring_prev(1);
     int *tmp = U; U = T; T = tmp;
     g.lvl = 0; g.deepest = 0; g.cur_is_a = 1;
@@ -542,9 +670,15 @@ struct Solver {
       g.deepest = g.lvl;
       int4 *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
       trace(2, g.nlen);
-      gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
+      if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited))
+        gr_level_bu<GRID>(g.lvl, base, nxt, ring_now(0), guard, gc);
+      else
+        gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
+      level_cols_flush();
       barrier<GRID>();
       g.nlen = (int)ring_prev(0);
+      g.fedges = ring_prev(4);
+      g.visited += ring_prev(5);
       g.cur_is_a ^= 1;
     }
     return true;
@@ -995,7 +1129,7 @@ struct Solver {
     // early stop (R22): every alive unmatched column is active; stop once all of them
     // carry a label.  alive unmatched = n - matched - dead; matched = m - |U|.
     c.gst.reached = (int)ring_prev(2);
-    c.gst.target = early_gr() ? n - (m - c.ulen) - (int)ld_rlx((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
+    c.gst.target = early_gr() ? n - (m - n_iso - c.ulen) - (int)ld_rlx((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
     if (c.gst.nlen == 0) gr_finish(c);
     else if (c.gst.reached >= c.gst.target) gr_finish(c, true);
     c.ns_gr += (long long)(tnow() - g0);
@@ -1012,8 +1146,14 @@ struct Solver {
     trace(2, g.nlen);
     const bool smemq = !GRID && p.tail_ctas == 1;
     if (smemq) tail_sq_begin(sfr(g.cur_is_a ? 1 : 0));
-    gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
+    if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited))
+      gr_level_bu<GRID>(g.lvl, c.base, nxt, ring_now(0), nullptr, &p.ctrl->gcnt);
+    else
+      gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
+    level_cols_flush();
     barrier<GRID>();
+    g.fedges = ring_prev(4);
+    g.visited += ring_prev(5);
     if (smemq) {
       tail_sq_end(g, nxt, sfr(g.cur_is_a ? 1 : 0));
     } else {
@@ -1128,7 +1268,8 @@ struct Solver {
         x->ho_ph = ph;
         const long long *src = reinterpret_cast<const long long *>(&c);
         for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) x->ho[j] = src[j];
-        for (int j = 0; j < 4; j++) x->ring[j][0] = x->ring[j][1] = x->ring[j][2] = x->ring[j][3] = 0;
+        for (int j = 0; j < 4; j++)
+          for (int q = 0; q < 8; q++) x->ring[j][q] = 0;
       }
     }
     grid_sync(&p.ctrl->bar, true);
@@ -1321,8 +1462,9 @@ struct Solver {
     int run1 = compact_pass1<true>(n, [&](int v) { return col_unmatched(v) ? v : -1; }, T, Ac);
     barrier<true>();
     int ulen = (int)ring_prev(0);
+    n_iso = (int)ring_prev(1);  // isolated rows (never in U)
     int len = compact_pass2<true>(n, T, Ac, run1, Ap);  // Ap = Ac (R12)
-    long long init_card = (long long)m - ulen;
+    long long init_card = (long long)m - n_iso - ulen;
 
     if (p.mode == MODE_GAP) {  // mcm_gap_relabel: labels in, labels out
       int gl = gap_relabel(1);
@@ -1443,11 +1585,10 @@ struct Solver {
 #ifndef MCM_MINB
 #define MCM_MINB 1
 #endif
-__global__ void __launch_bounds__(NT, MCM_MINB) gpr_kernel(Params p) {
-  extern __shared__ __align__(16) unsigned char smem_raw[];
-  Smem &sm = *reinterpret_cast<Smem *>(smem_raw);
-  Solver s(p, sm);
+__global__ void __launch_bounds__(NT, MCM_MINB) gpr_kernel(const __grid_constant__ Params p) {
+  Solver s(p);
   s.run();
 }
 
+#undef sm
 }  // namespace mcm

@@ -64,12 +64,15 @@ GR_GRAPHS = [
 ]
 
 
+@pytest.mark.parametrize("bu", [32, 0, 1], ids=["bu32", "topdown", "bottomup"])
 @pytest.mark.parametrize("gi", range(len(GR_GRAPHS)))
-def test_global_relabel_bit_exact(gi):
+def test_global_relabel_bit_exact(gi, bu):
+    """Top-down, bottom-up (direction-optimising) and mixed BFS levels must all give
+    the oracle's labels."""
     g = GR_GRAPHS[gi]()
     rng = np.random.default_rng(gi)
     ip, ix = dev(g)
-    mt = pkg.Matcher(ip, ix, g.m, g.n)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, bu_div=bu)
     for trial in range(3):
         if trial == 0:
             _, rm, cm = oracle.cheap_match(g)
@@ -108,7 +111,8 @@ OPTION_SETS = [
     dict(tail_max=0), dict(tail_max=100000), dict(grid_ctas=1), dict(grid_ctas=7), dict(gap=1), dict(tail_ctas=1),
     dict(tail_ctas=2), dict(tail_ctas=16), dict(compact_adapt=0), dict(grid_ctas=16, tail_ctas=16), dict(tail_f=64),
     dict(tail_max=4096, tail_f=100000), dict(tail_max=32, tail_f=32), dict(gr_early=1), dict(gr_early=1, tail_max=0),
-    dict(gr_early=1, k=3.0), dict(gr_early=0), dict(variant=1), dict(variant=1, gr_early=0, k=0.3),
+    dict(gr_early=1, k=3.0), dict(gr_early=0), dict(variant=1), dict(variant=1, gr_early=0, k=0.3), dict(bu_div=0),
+    dict(bu_div=1), dict(bu_div=100000),
 ]
 
 

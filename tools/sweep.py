@@ -41,17 +41,19 @@ def main():
     for spec in sys.argv[2:] or ["default"]:
         opts = parse(spec)
         mt = pkg.Matcher(ip, ix, g.m, g.n, **opts)
-        ts = []
+        ts, dev = [], []
         for r in range(reps):
             torch.cuda.synchronize()
             t0 = time.perf_counter()
             card, _, _ = mt.solve()
             ts.append((time.perf_counter() - t0) * 1e3)
+            dev.append(mt.stats()["ms_total"])
         st = mt.stats()
+        dev.sort()
         mt.close()
         keys = ["loops", "tail_loops", "gr_count", "gr_levels", "pushes", "blocked", "edges_scanned", "slots",
                 "grid_barriers", "ms_init", "ms_gr", "ms_loop", "ms_total"]
-        print(f"{name} {spec:30s} card={card} wall_ms={min(ts):8.3f} " +
+        print(f"{name} {spec:30s} card={card} dev_ms_med={dev[len(dev) // 2]:8.3f} min={dev[0]:8.3f} wall_ms={min(ts):8.3f} " +
               " ".join(f"{k}={st[k]:.3f}" if isinstance(st[k], float) else f"{k}={st[k]}" for k in keys), flush=True)
 
 
