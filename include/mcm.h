@@ -107,9 +107,13 @@ typedef struct {
                            order, needed for bit-exact serial runs); default 0 */
   int32_t bu_div;       /* direction-optimising GR: a BFS level whose frontier
                            has at least bu_div/8 adjacency entries per still-unlabelled
-                           column runs bottom-up (every unlabelled column looks for a
+                           column and at least n/64 rows runs bottom-up (every unlabelled
+                           column looks for a
                            neighbour at the current level); identical labels; default 16,
                            0 = top-down only */
+  int32_t scan_rot;     /* 1: every push scan starts at a (column, loop)-dependent rotation of
+                           Gamma(v) and wraps around -- a different but equally valid first
+                           minimum (reading R11); default 0 */
   int32_t variant;      /* 0 (default): G-PR (Alg. 7, active-column worklist);
                            1: G-PR-First (Alg. 3 + Alg. 6: every column
                            tested every loop; the Fig. 1 ablation) */

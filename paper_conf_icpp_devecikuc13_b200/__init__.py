@@ -51,6 +51,7 @@ class Options(ctypes.Structure):
         ("serial", ctypes.c_int32),
         ("sort_csc", ctypes.c_int32),
         ("bu_div", ctypes.c_int32),
+        ("scan_rot", ctypes.c_int32),
         ("variant", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]

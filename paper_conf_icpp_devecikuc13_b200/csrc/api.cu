@@ -371,6 +371,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.serial = o.serial;
   p.variant = o.variant;
   p.bu_div = o.bu_div;
+  p.scan_rot = o.serial ? 0 : o.scan_rot;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either
     p.tail_max = 0;
     p.serial = 0;

@@ -79,7 +79,8 @@ struct Params {
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
-  int bu_div;              // bottom-up BFS level when frontier * bu_div >= n (0: top-down only)
+  int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
+  int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -604,8 +605,8 @@ struct Solver {
   // bottom-up when the frontier's adjacency entries reach bu_div/8 times the
   // columns still unlabelled (Beamer-style edge rule; frontier rows alone mislead on
   // low-degree road graphs)
-  __device__ __forceinline__ bool use_bottom_up(long long fedges, long long unvisited) const {
-    return p.bu_div > 0 && fedges * 8 >= unvisited * (long long)p.bu_div;
+  __device__ __forceinline__ bool use_bottom_up(long long fedges, long long unvisited, int nlen) const {
+    return p.bu_div > 0 && fedges * 8 >= unvisited * (long long)p.bu_div && (long long)nlen * 64 >= n;
   }
 
   u32 gr_base = 0;
@@ -670,7 +671,7 @@ struct Solver {
       g.deepest = g.lvl;
       int4 *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
       trace(2, g.nlen);
-      if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited))
+      if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited, g.nlen))
         gr_level_bu<GRID>(g.lvl, base, nxt, ring_now(0), guard, gc);
       else
         gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
@@ -760,6 +761,7 @@ struct Solver {
         if (p.dead_skip && psiv >= INF) e = s;  // R19: provably unmatchable
       }
       const int target = psiv - 1;
+      const int rot = (p.scan_rot && e - s > 1) ? (int)(((u32)v * 2654435761u + (u32)loop * 2246822519u) % (u32)(e - s)) : 0;
       bool huge = v >= 0 && e - s > HUGE_DEG;
       if (huge && gl == 0) {  // defer to the CTA-wide pass below
         int q = atomicAdd(&sm.nhuge, 1);
@@ -770,16 +772,17 @@ struct Solver {
       const bool big = v >= 0 && !huge && G < 32 && e - s > BIG_DEG;
       u64 best = ~0ull;
       int ub = -1, wb = -1;
-      if (v >= 0 && !big && !huge) scan(s, e, gl, G, gmask, target, base, best, ub, wb);  // l.6-11
+      if (v >= 0 && !big && !huge) scan(s, e, gl, G, gmask, target, base, best, ub, wb, rot);  // l.6-11
       unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
       while (bigm) {  // long lists: the whole warp
         int bl = __ffs(bigm) - 1;
         bigm &= bigm - 1;
         int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
         int tb = __shfl_sync(0xffffffffu, target, bl);
+        int rb = __shfl_sync(0xffffffffu, rot, bl);
         u64 b2;
         int u2, w2;
-        scan(sb, eb, lane, 32, 0xffffffffu, tb, base, b2, u2, w2);
+        scan(sb, eb, lane, 32, 0xffffffffu, tb, base, b2, u2, w2, rb);
         if (lane == bl) { best = b2; ub = u2; wb = w2; }
       }
       if (gl == 0 && !huge) {
@@ -863,18 +866,24 @@ struct Solver {
   // l.6-11): the G lanes of a group read KB*G consecutive neighbours per step, take
   // the (label, position) minimum and stop after the step in which the running
   // minimum reaches psi(v)-1 (reading R11).  best = (label << 32 | position) or ~0.
+  // rot: the scan starts at position s + rot and wraps around (option scan_rot, a
+  // free tie-break in parallel mode, R11: contenders for one low-label row spread
+  // over the equally low rows instead of blocking each other)
   __device__ __forceinline__ void scan(int s, int e, int gl, int G, unsigned gmask, int target, u32 base, u64 &best,
-                                       int &bu, int &bw) {
+                                       int &bu, int &bw, int rot = 0) {
     best = ~0ull;
     bu = -1;
     bw = -1;
+    const int len = e - s;
     for (int c0 = s; c0 < e; c0 += G * KB) {
       int x[KB];
       u64 rs[KB];
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         int jj = c0 + gl + k * G;
-        x[k] = jj < e ? ld_ro(p.cadj + jj) : -1;
+        int q = jj - s + rot;
+        if (q >= len) q -= len;
+        x[k] = jj < e ? ld_ro(p.cadj + s + q) : -1;
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
@@ -1146,7 +1155,7 @@ struct Solver {
     trace(2, g.nlen);
     const bool smemq = !GRID && p.tail_ctas == 1;
     if (smemq) tail_sq_begin(sfr(g.cur_is_a ? 1 : 0));
-    if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited))
+    if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited, g.nlen))
       gr_level_bu<GRID>(g.lvl, c.base, nxt, ring_now(0), nullptr, &p.ctrl->gcnt);
     else
       gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
