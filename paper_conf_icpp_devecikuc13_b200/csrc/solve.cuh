@@ -1296,7 +1296,7 @@ struct Solver {
 
   // Serial mode (tests): one thread runs the fix and push steps of Alg. 7 with the
   // slots in increasing order -- exactly the schedule of the oracle's serial
-  // simulator (oracle.c or_gpr_serial) -- until a GR (which runs on the grid, as
+  // simulator (or_gpr_serial, test side) -- until a GR (which runs on the grid, as
   // always) or a gap relabel is due, or no active column is left.  Trajectory,
   // matching and counters are then bit-exact against the simulator.
   __device__ void serial_fix_push(Ctl &c, int &reason) {
