@@ -273,8 +273,9 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   CK(cudaGetDevice(&h->dev));
   CK(cudaDeviceGetAttribute(&h->sms, cudaDevAttrMultiProcessorCount, h->dev));
   int per_sm = 0;
-  CK(cudaFuncSetAttribute(gpr_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Smem)));
-  CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel, NT, sizeof(Smem)));
+  CK(cudaFuncSetAttribute(gpr_kernel<F_FAST>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Smem)));
+  CK(cudaFuncSetAttribute(gpr_kernel<F_ALL>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(Smem)));
+  CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gpr_kernel<F_ALL>, NT, sizeof(Smem)));
   if (per_sm < 1) return MCM_EINTERNAL;
   h->max_grid = h->sms * (per_sm > 2 ? 2 : per_sm);  // one or two CTAs per SM (MCM_MINB)
   if (h->max_grid > MAX_CTAS) h->max_grid = MAX_CTAS;
@@ -385,12 +386,15 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
+  // the lean production instance unless a feature only the full one carries is on
+  void (*kern)(const Params) =
+      (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug) ? gpr_kernel<F_ALL> : gpr_kernel<F_FAST>;
   int C = o.tail_ctas;
   if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
   int maxg = h->max_grid;
   if (C > 1) {
     // co-resident clusters of C CTAs (the tail group is cluster 0)
-    if (C > 8) CK(cudaFuncSetAttribute(gpr_kernel, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    if (C > 8) CK(cudaFuncSetAttribute(kern, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
     cudaLaunchConfig_t q = {};
     cudaLaunchAttribute qa[1];
     qa[0].id = cudaLaunchAttributeClusterDimension;
@@ -398,7 +402,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     q.gridDim = dim3(C); q.blockDim = dim3(NT); q.attrs = qa; q.numAttrs = 1;
     q.dynamicSmemBytes = sizeof(Smem);
     int ncl = 0;
-    CK(cudaOccupancyMaxActiveClusters(&ncl, gpr_kernel, &q));
+    CK(cudaOccupancyMaxActiveClusters(&ncl, kern, &q));
     if (ncl < 1) return MCM_EINTERNAL;
     maxg = std::min(maxg, ncl * C);
   }
@@ -416,7 +420,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   at[1].val.clusterDim.x = C; at[1].val.clusterDim.y = 1; at[1].val.clusterDim.z = 1;
   cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = sizeof(Smem); cfg.stream = st;
   cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
-  CK(cudaLaunchKernelEx(&cfg, gpr_kernel, p));
+  CK(cudaLaunchKernelEx(&cfg, kern, p));
   CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));
   CK(cudaStreamSynchronize(st));
   const Ctrl &c = h->host_ctrl;

@@ -17,6 +17,9 @@
 
 namespace cg = cooperative_groups;
 
+#ifndef MCM_FINE
+#define MCM_FINE 0
+#endif
 namespace mcm {
 
 constexpr int NT = 512;          // threads per CTA
@@ -87,9 +90,25 @@ struct Params {
   int *rmatch_out, *cmatch_out;  // solve: matching; relabel: psi_row / psi_col
 };
 
+// per-CTA statistics accumulators (Smem::st), flushed at every barrier from
+// per-thread 32-bit counters that live only within one phase
+enum { SS_PUSH, SS_BLOCK, SS_DEAD, SS_SCAN, SS_SLOTS, SS_FREE, SS_GRROWS, SS_GREDGES, SS_GRCOLS, SS_GYEDGES, SS_N };
+// control-loop statistics and the phase-trace cursor: kept by the lead thread
+// (block 0, thread 0) only, in shared memory, so they hold no registers
+struct LeadStats {
+  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar;
+  int tn, ttag, tsz, pad;
+};
 struct Smem;
 extern __shared__ Smem smem_dyn[];
 struct Smem {
+  u32 ts[SS_N][NT];        // per-thread statistics (thread-private slots: no atomics)
+  LeadStats ld;
+  u32 lvc[2];              // BFS level: [1] next-frontier adjacency entries (direction choice)
+  u32 rp[8];               // phase counters of the last completed phase (loaded by thread 0)
+  u32 bc;                  // broadcast slot (bcast_ld)
+  int ho_reason, ho_ph;    // tail hand-over image (loaded by thread 0 after the barrier)
+  long long ho[32];
   long long red[NWARP];
   int w[NWARP];
   alignas(16) int q[QCAP];
@@ -113,6 +132,16 @@ __device__ __forceinline__ u64 gtime() {
 // phase timers: only the lead thread (block 0, thread 0) reads the clock
 __device__ __forceinline__ u64 tnow() { return (threadIdx.x == 0 && blockIdx.x == 0) ? gtime() : 0ull; }
 
+// Compile-time feature set of a kernel instance.  The production solve kernel
+// carries only what a default solve runs; the test / ablation / auxiliary paths
+// (serial mode, G-PR-First, debug checks, gap relabelling, the label-only modes)
+// live in a second instance, so they cost the hot kernel no code size (its
+// instruction footprint is on the critical path of every short phase).
+enum { F_SERIAL = 1, F_FIRST = 2, F_DEBUG = 4, F_GAP = 8, F_AUX = 16, F_BU = 32 };
+constexpr int F_FAST = F_BU;
+constexpr int F_ALL = F_SERIAL | F_FIRST | F_DEBUG | F_GAP | F_AUX | F_BU;
+
+template <int F>
 struct Solver {
   const Params &p;
   // the dynamic shared block, named through a namespace-scope extern __shared__
@@ -120,21 +149,23 @@ struct Solver {
   // made the staging atomics generic ATOM.E)
 #define sm (smem_dyn[0])
   const int m, n, INF;
-  // per-thread statistics (reduced at the end)
-  long long s_push = 0, s_block = 0, s_dead = 0, s_scan = 0, s_slots = 0, s_free = 0;
-  long long s_grrows = 0, s_gredges = 0, s_grcols = 0, s_gyedges = 0, s_gapkill = 0;
+  // per-thread statistics: 32-bit thread-private slots in shared memory (Smem::ts),
+  // summed at the end of the solve -- they hold no registers, need no atomics and
+  // no per-phase reduction (a per-phase warp flush with 64-bit shared atomics, which
+  // are CAS spin loops on sm_100, cost ~1 us per BFS level)
   int ph = 0;  // phase counter: identical in every thread
-  long long nbar = 0;
-  int ttag = 0, tsz = 0, tn = 0;  // phase trace (lead thread only)
-  long long gaps_total = 0;
+  __device__ __forceinline__ static bool lead() { return threadIdx.x == 0 && blockIdx.x == 0; }
+  __device__ __forceinline__ static LeadStats &L() { return smem_dyn[0].ld; }
+  __device__ __forceinline__ static u32 &S(int k) { return smem_dyn[0].ts[k][threadIdx.x]; }
   __device__ __forceinline__ void trace(int tag, int sz) {
-    ttag = tag; tsz = sz;
+    if (lead()) { L().ttag = tag; L().tsz = sz; }
   }
-  // extra trace point (no barrier): lead thread only
-  __device__ __forceinline__ void tmark(int tag, int sz) {
-    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
+  __device__ __forceinline__ void tmark(int tag, int sz) { trace_rec(tag, sz); }
+  __device__ __forceinline__ void trace_rec(int tag, int sz) {
+    if (p.trace && lead() && L().tn < p.trace_cap) {
+      const int tn = L().tn;
       p.trace[3 * tn] = tag; p.trace[3 * tn + 1] = sz; p.trace[3 * tn + 2] = (long long)gtime();
-      tn++;
+      L().tn = tn + 1;
     }
   }
 
@@ -148,24 +179,37 @@ struct Solver {
   // ring[ph & 3] collects the counts produced during phase ph; the consumer reads
   // it right after the barrier.  ring[(ph + 2) & 3] was produced two phases ago
   // and consumed at the start of the previous phase, so CTA 0 may clear it now.
-  template <bool GRID>
+  // RP: the next phase reads the counters of this one (ring_prev); loading them
+  // is one more L2 round trip on the barrier's critical path, so barriers whose
+  // successor does not need them skip it
+  template <bool GRID, bool RP = true>
   __device__ __forceinline__ void barrier() {
+    const u32 *rn = p.ctrl->ring[ph & 3];
+    auto load_rp = [&] {
+#pragma unroll
+      for (int j = 0; j < 8; j++) sm.rp[j] = ld_rlx(rn + j);
+    };
     if (GRID) {
-      grid_sync(&p.ctrl->bar, false);
-      nbar++;
-    } else if (p.tail_ctas > 1) {
-      // tail group = thread-block cluster 0: hardware cluster barrier (release /
-      // acquire at cluster scope covers the global writes of the cluster's CTAs)
-      asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
+      if (MCM_FINE) tmark(105, 0);
+      if (RP) grid_sync(&p.ctrl->bar, false, load_rp);
+      else grid_sync(&p.ctrl->bar, false);
+      if (lead()) L().nbar++;
     } else {
-      __syncthreads();
+      if (p.tail_ctas > 1) {
+        // tail group = thread-block cluster 0: hardware cluster barrier (release /
+        // acquire at cluster scope covers the global writes of the cluster's CTAs)
+        asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
+      } else {
+        __syncthreads();
+      }
+      if (RP) {
+        if (threadIdx.x < 8) sm.rp[threadIdx.x] = ld_rlx(rn + threadIdx.x);
+        __syncthreads();
+      }
     }
     // phase trace: stamped after the barrier, so a phase's duration includes its
     // slowest CTA
-    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
-      p.trace[3 * tn] = ttag * 2 + (GRID ? 1 : 0); p.trace[3 * tn + 1] = tsz; p.trace[3 * tn + 2] = (long long)gtime();
-      tn++;
-    }
+    if (p.trace && lead()) trace_rec(L().ttag * 2 + (GRID ? 1 : 0), L().tsz);
     ph++;
     if (blockIdx.x == 0 && threadIdx.x == 0) {
       u32 *r = p.ctrl->ring[(ph + 2) & 3];
@@ -174,7 +218,15 @@ struct Solver {
     }
   }
   __device__ __forceinline__ u32 *ring_now(int j) { return &p.ctrl->ring[ph & 3][j]; }
-  __device__ __forceinline__ u32 ring_prev(int j) { return ld_rlx(&p.ctrl->ring[(ph - 1) & 3][j]); }
+  // counter j of the phase completed by the last barrier (every barrier loads them)
+  __device__ __forceinline__ u32 ring_prev(int j) const { return sm.rp[j]; }
+  // a CTA-uniform global word, loaded once per CTA
+  __device__ __forceinline__ u32 bcast_ld(const u32 *a) {
+    __syncthreads();
+    if (threadIdx.x == 0) sm.bc = ld_rlx(a);
+    __syncthreads();
+    return sm.bc;
+  }
 
   template <bool GRID>
   __device__ __forceinline__ int cta() const { return blockIdx.x; }  // tail group = blocks [0, tail_ctas)
@@ -237,10 +289,18 @@ struct Solver {
       next[sm.qbase + c + j] = q;
       fe += (u32)(q.z - q.y);
     }
-    fe = __reduce_add_sync(0xffffffffu, fe);
-    if (lane_id() == 0 && fe) atomicAdd(ring_now(4), fe);
+    if (fe_on) {  // the CTA's sum rides on the two barriers below
+      fe = __reduce_add_sync(0xffffffffu, fe);
+      if (lane_id() == 0 && fe) atomicAdd(&sm.lvc[1], fe);
+    }
     __syncthreads();
-    if (threadIdx.x == 0) sm.qcnt = 0;
+    if (threadIdx.x == 0) {
+      sm.qcnt = 0;
+      if (fe_on && sm.lvc[1]) {
+        atomicAdd(ring_now(4), sm.lvc[1]);
+        sm.lvc[1] = 0;
+      }
+    }
     __syncthreads();
   }
 
@@ -249,8 +309,8 @@ struct Solver {
   // or -1.  Survivors of CTA c's chunk go to T[lo_c + rank]; ctacnt[c] = count.
   // GRID=false: a single CTA, written straight to `out` (reads of a tile finish
   // before its writes, and writes never pass the tile being read).
-  template <bool GRID, class F>
-  __device__ int compact_pass1(int len, F f, int *T, int *out) {
+  template <bool GRID, class Fn>
+  __device__ int compact_pass1(int len, Fn f, int *T, int *out) {
     const int C = ncta<GRID>(), c = cta<GRID>();
     const int chunk = (len + C - 1) / C;
     const int lo = min(len, c * chunk), hi = min(len, lo + chunk);
@@ -343,7 +403,7 @@ struct Solver {
 #pragma unroll
           for (int k = 0; k < KB; k++) {
             if (done || u[k] < 0) continue;
-            s_gyedges++;
+            S(SS_GYEDGES)++;
             if (mu_of(rs[k]) != -1) continue;
             if (atomicCAS(p.rowst + u[k], rs[k], pack(v, psi_of(rs[k]))) == rs[k]) {
               st_rlx(p.colst + v, pack(u[k], 0));
@@ -363,7 +423,7 @@ struct Solver {
           int j = c0 + lane;
           int u = -1;
           u64 rs = 0;
-          if (j < eb) { u = ld_ro(p.cadj + j); rs = ld_rlx(p.rowst + u); s_gyedges++; }
+          if (j < eb) { u = ld_ro(p.cadj + j); rs = ld_rlx(p.rowst + u); S(SS_GYEDGES)++; }
           unsigned cand = __ballot_sync(0xffffffffu, u >= 0 && mu_of(rs) == -1);
           while (cand && !done) {
             int l = __ffs(cand) - 1;
@@ -428,6 +488,7 @@ struct Solver {
     const u32 lc = base + lvl + 1, lr = base + lvl + 2;
     const int G = pick_group(curlen, ncta<GRID>() * NT);
     const int gl = lane & (G - 1), per_tile = NT / G;
+    if (GRID && lvl > 0 && MCM_FINE) tmark(101, curlen);
     for (int t = cta<GRID>() * per_tile; t < curlen; t += ncta<GRID>() * per_tile) {
       int i = t + (int)threadIdx.x / G;
       int u = -1, s = 0, e = 0;
@@ -451,7 +512,8 @@ struct Solver {
         int4 q = ld_q(cur4 + i);
         u = q.x; s = q.y; e = q.z;
       }
-      if (u >= 0 && gl == 0) { s_grrows++; s_gredges += e - s; }
+      if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(102, 0);
+      if (u >= 0 && gl == 0) { S(SS_GRROWS)++; S(SS_GREDGES) += e - s; }
       const bool big = u >= 0 && G < 32 && e - s > BIG_DEG;
       if (u >= 0 && !big) expand(s + gl, e, G, lc, lr, next, ncnt, guard, gcnt, G >= 4);
       unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
@@ -461,7 +523,9 @@ struct Solver {
         int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
         expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt, false);
       }
+      if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(103, 0);
       flush(next, ncnt);
+      if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(104, 0);
     }
   }
   // Visit radj[j], j = j0, j0+step, ... < e, KB at a time.  A CAS claims each
@@ -512,14 +576,13 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         if (old[k] != cs[k]) continue;  // not claimed by this thread
-        s_grcols++;
-        lvl_cols++;
+        S(SS_GRCOLS)++;
         int w = mu_of(cs[k]);
         if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: mu(v) > -1 and mu(mu(v)) = v
           st_rlx(p.rowst + w, pack(v[k], lr));
           stage(make_int4(w, rs[k], re[k], 0), next, ncnt);
         } else {
-          s_free++;
+          S(SS_FREE)++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
           if (mu_of(cs[k]) != -2) atomicAdd(ring_now(2), 1u);  // an alive unmatched column got its label
         }
@@ -561,7 +624,7 @@ struct Solver {
           for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
 #pragma unroll
           for (int k = 0; k < KB; k++) hit |= x[k] >= 0 && psi_of(rs[k]) == lf;
-          s_gredges += min(KB, e - j);
+          S(SS_GREDGES) += min(KB, e - j);
         }
       }
       unsigned bigm = __ballot_sync(0xffffffffu, open && e - s > BIG_DEG);
@@ -578,14 +641,13 @@ struct Solver {
             if (jj < eb) h |= psi_of(ld_rlx(p.rowst + ld_ro(p.cadj + jj))) == lf;
           }
           any = __any_sync(0xffffffffu, h);
-          if (lane == 0) s_gredges += min(32 * KB, eb - c0);
+          if (lane == 0) S(SS_GREDGES) += min(32 * KB, eb - c0);
         }
         if (lane == bl) hit = any;
       }
       if (hit) {
         st_rlx(p.colst + v, pack(mu_of(cs), lc));
-        s_grcols++;
-        lvl_cols++;
+        S(SS_GRCOLS)++;
         const int w = mu_of(cs);
         u64 rw = 0;
         int rs = 0, re = 0;
@@ -594,7 +656,7 @@ struct Solver {
           st_rlx(p.rowst + w, pack(v, lr));
           stage(make_int4(w, rs, re, 0), next, ncnt);
         } else {
-          s_free++;
+          S(SS_FREE)++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v;
           if (w != -2) atomicAdd(ring_now(2), 1u);
         }
@@ -606,15 +668,18 @@ struct Solver {
   // columns still unlabelled (Beamer-style edge rule; frontier rows alone mislead on
   // low-degree road graphs)
   __device__ __forceinline__ bool use_bottom_up(long long fedges, long long unvisited, int nlen) const {
-    return p.bu_div > 0 && fedges * 8 >= unvisited * (long long)p.bu_div && (long long)nlen * 64 >= n;
+    return (F & F_BU) && p.bu_div > 0 && fedges * 8 >= unvisited * (long long)p.bu_div && (long long)nlen * 64 >= n;
   }
 
   u32 gr_base = 0;
-  u32 lvl_cols = 0;  // columns this thread labelled in the current level
-  __device__ __forceinline__ void level_cols_flush() {
-    u32 x = __reduce_add_sync(0xffffffffu, lvl_cols);
-    if (lane_id() == 0 && x) atomicAdd(ring_now(5), x);
-    lvl_cols = 0;
+  // Direction choice bookkeeping (bottom-up BFS levels): the adjacency entries of
+  // the next frontier (ring counter 4) are summed only when the current frontier is
+  // within a factor 4 of the bottom-up size threshold (flush, fe_on); the columns
+  // labelled so far follow from counters the level produces anyway (next-frontier
+  // rows + reached unmatched columns), so narrow levels pay nothing for it.
+  bool fe_on = false;
+  __device__ __forceinline__ void set_fe(long long nlen) {
+    fe_on = (F & F_BU) && p.bu_div > 0 && nlen * 256 >= n;
   }
   int fl_r = 0, fl_c = 0;  // push: labels of vertices the last GR did not reach (set from Ctl)
   __device__ __forceinline__ int labf(u32 s, u32 base, int stale) const {
@@ -633,7 +698,7 @@ struct Solver {
     GRState g;
     gr_start<GRID>(g, U, ulen, T, Qa, base, guard);
     gr_levels<GRID>(g, base, Qa, Qb, guard, 0x7fffffff);
-    gcount = (int)ld_rlx(&p.ctrl->gcnt);
+    gcount = (int)bcast_ld(&p.ctrl->gcnt);
     return g.deepest + 2;
   }
 
@@ -649,12 +714,12 @@ struct Solver {
     gr_base = base;
     u32 *gc = &p.ctrl->gcnt;  // zero here: reset one phase after its last use
     trace(1, ulen);
+    set_fe(ulen);
     gr_level<GRID>(U, nullptr, ulen, 0, base, Qa, ring_now(0), T, ring_now(1), guard, gc);
-    level_cols_flush();
     barrier<GRID>();
     g.nlen = (int)ring_prev(0);
     g.fedges = ring_prev(4);
-    g.visited = ring_prev(5);
+    g.visited = (long long)g.nlen + ring_prev(2);
     ulen = (int)ring_prev(1);
     int *tmp = U; U = T; T = tmp;
     g.lvl = 0; g.deepest = 0; g.cur_is_a = 1;
@@ -671,15 +736,15 @@ struct Solver {
       g.deepest = g.lvl;
       int4 *cur = g.cur_is_a ? Qa : Qb, *nxt = g.cur_is_a ? Qb : Qa;
       trace(2, g.nlen);
+      set_fe(g.nlen);
       if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited, g.nlen))
         gr_level_bu<GRID>(g.lvl, base, nxt, ring_now(0), guard, gc);
       else
         gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, base, nxt, ring_now(0), nullptr, nullptr, guard, gc);
-      level_cols_flush();
       barrier<GRID>();
       g.nlen = (int)ring_prev(0);
       g.fedges = ring_prev(4);
-      g.visited += ring_prev(5);
+      g.visited += (long long)g.nlen + ring_prev(2);
       g.cur_is_a ^= 1;
     }
     return true;
@@ -709,7 +774,7 @@ struct Solver {
       int i = t + threadIdx.x;
       if (i < len) cnt += fix_slot(i, Ac, Ap, loop) != -1;
     }
-    s_slots += cnt;
+    S(SS_SLOTS) += cnt;
     add_count(cnt, j);
   }
 
@@ -728,16 +793,16 @@ struct Solver {
         st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
         st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
         Ap[i] = wb;                                     // l.18 (R3)
-        s_push++;
+        S(SS_PUSH)++;
       } else {
         Ap[i] = -1;                                     // R4: blocked
-        s_block++;
+        S(SS_BLOCK)++;
       }
     } else {
       st_rlx(p.colst + v, pack(-2, psi_of(cs)));        // l.20
       Ac[i] = -1;                                       // l.21
       Ap[i] = -1;                                       // l.22
-      s_dead++;
+      S(SS_DEAD)++;
       atomicAdd(&p.ctrl->ndead, 1u);
     }
   }
@@ -834,7 +899,7 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         if (x[k] < 0) continue;
-        s_scan++;
+        S(SS_SCAN)++;
         int l = labf(psi_of(rs[k]), base, fl_r);
         u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + (int)threadIdx.x + k * NT - s)) : ~0ull;
         if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
@@ -892,7 +957,7 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         if (x[k] < 0) continue;
-        s_scan++;
+        S(SS_SCAN)++;
         int l = labf(psi_of(rs[k]), base, fl_r);
         u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + gl + k * G - s)) : ~0ull;
         if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
@@ -953,20 +1018,20 @@ struct Solver {
   }
   // rows: mu(u) = v >= 0  =>  mu(v) = u ;  worklist: no column twice
   __device__ void debug_check(int where, long long loop, const int *Ac, int len) {
-    if (!p.debug) return;
+    if (!(F & F_DEBUG) || !p.debug) return;
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     for (int u = g; u < m; u += G) {
       int c = mu_of(ld_rlx(p.rowst + u));
       if (c >= 0 && mu_of(ld_rlx(p.colst + c)) != u) dbg_record(where, loop, u, c);
     }
     for (int v = g; v < n; v += G) p.dbgbuf[v] = 0;
-    barrier<true>();
+    barrier<true, false>();
     if (Ac)
       for (int i = g; i < len; i += G) {
         int v = __ldcg(Ac + i);
         if (v >= 0 && atomicAdd(p.dbgbuf + v, 1) != 0) dbg_record(100 + where, loop, v, i);
       }
-    barrier<true>();
+    barrier<true, false>();
   }
 
   // ---------------------------------------------------------------- gap relabel
@@ -1006,15 +1071,15 @@ struct Solver {
     if (threadIdx.x == 0) sm.qcnt = 0;
     for (int o = 16; o > 0; o >>= 1) lmax = max(lmax, __shfl_xor_sync(0xffffffffu, lmax, o));
     if (lane_id() == 0 && lmax >= 0) atomicMax(&c->gmax, lmax);
-    barrier<true>();
-    const int L = min((int)ld_rlx((const u32 *)&c->gmax), H);
+    barrier<true, false>();
+    const int L = min((int)bcast_ld((const u32 *)&c->gmax), H);
     int first = 0x7fffffff;
     for (int l = g; l < L; l += G)
       if (__ldcg(p.hist + l) == 0) { first = l; break; }
     for (int o = 16; o > 0; o >>= 1) first = min(first, __shfl_xor_sync(0xffffffffu, first, o));
     if (lane_id() == 0 && first != 0x7fffffff) atomicMin(&c->gmin, first);
-    barrier<true>();
-    const int gap = (int)ld_rlx((const u32 *)&c->gmin);
+    barrier<true, false>();
+    const int gap = (int)bcast_ld((const u32 *)&c->gmin);
     if (blockIdx.x == 0 && threadIdx.x == 0) c->gmax = 0;
     long long killed = 0;
     if (gap != 0x7fffffff) {
@@ -1026,8 +1091,7 @@ struct Solver {
       }
     }
     for (int l = g; l < L; l += G) p.hist[l] = 0;
-    s_gapkill += killed;
-    barrier<true>();
+    barrier<true, false>();
     return gap == 0x7fffffff ? -1 : gap;
   }
 
@@ -1041,8 +1105,6 @@ struct Solver {
     int shrink, compact_next, gr_active, ac0, u0, pad;
     int floor_r, floor_c;  // labels of vertices the last GR did not reach (m+n unless it stopped early)
     GRState gst;
-    // statistics (meaningful in the lead thread)
-    long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop;
   };
   static_assert(sizeof(Ctl) % 8 == 0 && sizeof(Ctl) / 8 <= 32, "Ctl handoff image");
   __device__ __forceinline__ int *Acp(const Ctl &c) const { return c.ac0 ? p.wl0 : p.wl1; }
@@ -1058,7 +1120,7 @@ struct Solver {
   enum { R_NONE = 0, R_TERM = 1, R_GRID = 2, R_CAP = 4 };
   // gap relabel schedule (R14): once, halfway between two GRs
   __device__ __forceinline__ long long gap_at(long long loop, long long iterGR) const {
-    return (p.gap && iterGR - loop >= 2) ? loop + (iterGR - loop) / 2 : -1;
+    return ((F & F_GAP) && p.gap && iterGR - loop >= 2) ? loop + (iterGR - loop) / 2 : -1;
   }
   // GR frontiers of at most tail_f() rows run on the tail group (hand-over back to
   // the grid when a frontier outgrows it, back to the tail below tail_f()/2)
@@ -1112,8 +1174,7 @@ struct Solver {
     c.floor_r = early ? c.gst.lvl + 4 : INF;
     if (early) c.gst.deepest = c.gst.lvl + 2;
     int ml = c.gst.deepest + 2;
-    c.grs++;
-    c.levels += ml / 2;
+    if (lead()) { L().grs++; L().levels += ml / 2; }
     c.iterGR = c.loop + iter_gap(ml);
     c.gapAt = gap_at(c.loop, c.iterGR);
     c.shrink = 1;
@@ -1138,15 +1199,16 @@ struct Solver {
     // early stop (R22): every alive unmatched column is active; stop once all of them
     // carry a label.  alive unmatched = n - matched - dead; matched = m - |U|.
     c.gst.reached = (int)ring_prev(2);
-    c.gst.target = early_gr() ? n - (m - n_iso - c.ulen) - (int)ld_rlx((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
+    c.gst.target = early_gr() ? n - (m - n_iso - c.ulen) - (int)bcast_ld((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
     if (c.gst.nlen == 0) gr_finish(c);
     else if (c.gst.reached >= c.gst.target) gr_finish(c, true);
-    c.ns_gr += (long long)(tnow() - g0);
+    if (lead()) L().ns_gr += (long long)(tnow() - g0);
   }
   // one BFS level (Alg. 5)
   template <bool GRID>
   __device__ void gr_step(Ctl &c) {
     u64 g0 = tnow();
+    if (GRID && MCM_FINE) tmark(107, 0);
     GRState &g = c.gst;
     g.lvl += 2;
     g.deepest = g.lvl;
@@ -1155,14 +1217,13 @@ struct Solver {
     trace(2, g.nlen);
     const bool smemq = !GRID && p.tail_ctas == 1;
     if (smemq) tail_sq_begin(sfr(g.cur_is_a ? 1 : 0));
+    set_fe(g.nlen);
     if (GRID && use_bottom_up(g.fedges, (long long)n - g.visited, g.nlen))
       gr_level_bu<GRID>(g.lvl, c.base, nxt, ring_now(0), nullptr, &p.ctrl->gcnt);
     else
       gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
-    level_cols_flush();
     barrier<GRID>();
     g.fedges = ring_prev(4);
-    g.visited += ring_prev(5);
     if (smemq) {
       tail_sq_end(g, nxt, sfr(g.cur_is_a ? 1 : 0));
     } else {
@@ -1171,9 +1232,11 @@ struct Solver {
     }
     g.cur_is_a ^= 1;
     g.reached += (int)ring_prev(2);
+    g.visited += (long long)g.nlen + ring_prev(2);
     if (g.nlen == 0) gr_finish(c);
     else if (g.reached >= g.target) gr_finish(c, true);
-    c.ns_gr += (long long)(tnow() - g0);
+    if (GRID && MCM_FINE) tmark(106, 0);
+    if (lead()) L().ns_gr += (long long)(tnow() - g0);
   }
   // one iteration of Alg. 7 l.10-19: fix step (INITKRNL, or SHRKRNL = fix + stable
   // compaction), then PUSHKRNL and the Ac/Ap swap.  Returns false when the fix
@@ -1186,17 +1249,17 @@ struct Solver {
     int act;
     trace(3, c.len);
     if (!GRID || (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) || p.compact_every || c.compact_next) {
-      if (threadIdx.x == 0 && (GRID ? blockIdx.x == 0 : true)) s_slots += c.len;
+      if (lead()) S(SS_SLOTS) += c.len;
       int r1 = compact_pass1<GRID>(c.len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, Tb(c), Ac);
-      barrier<GRID>();
+        barrier<GRID, false>();
       if (ncta<GRID>() > 1) {
         c.len = compact_pass2<GRID>(c.len, Tb(c), Ac, r1);
-        barrier<GRID>();  // Ac was rewritten by other CTAs: order it before PUSH
+        barrier<GRID, false>();  // Ac was rewritten by other CTAs: order it before PUSH
       } else {
         c.len = r1;
       }
       act = c.len;
-      if (c.shrink) c.shrinks++;
+      if (c.shrink && lead()) L().shrinks++;
       c.shrink = 0;
       c.compact_next = 0;
     } else {
@@ -1209,19 +1272,19 @@ struct Solver {
     }
     if (GRID) debug_check(3, c.loop, Ac, c.len);
     if (act == 0) {
-      c.ns_loop += (long long)(tnow() - l0);
+      if (lead()) L().ns_loop += (long long)(tnow() - l0);
       return false;
     }
     trace(4, c.len);
     fl_r = c.floor_r;
     fl_c = c.floor_c;
     push<GRID>(c.len, Ac, Ap, lp, cur);
-    barrier<GRID>();
+    barrier<GRID, false>();
     if (GRID) debug_check(4, c.loop, nullptr, 0);
     c.ac0 ^= 1;  // l.18: swap Ac and Ap
     c.loop++;    // l.19
-    if (GRID) c.loops++; else c.tail_loops++;
-    c.ns_loop += (long long)(tnow() - l0);
+    if (lead()) { if (GRID) L().loops++; else L().tail_loops++; }
+    if (lead()) L().ns_loop += (long long)(tnow() - l0);
     return true;
   }
 
@@ -1233,6 +1296,19 @@ struct Solver {
   // (P:525-528).  It stops when a unit needs the grid (R_GRID), when no active
   // column is left (R_TERM) or at the iteration cap (R_CAP), publishes its Ctl and
   // every CTA adopts it after the barrier.
+  // thread 0, after the barrier: the published hand-over image -> shared memory
+  __device__ __forceinline__ void load_handover() {
+    const Ctrl *x = p.ctrl;
+    sm.ho_reason = (int)ld_rlx((const u32 *)&x->ho_reason);
+    sm.ho_ph = (int)ld_rlx((const u32 *)&x->ho_ph);
+#pragma unroll
+    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) sm.ho[j] = ld_rlx(&x->ho[j]);
+  }
+  __device__ __forceinline__ void adopt_handover(Ctl &c) {
+    long long *dst = reinterpret_cast<long long *>(&c);
+#pragma unroll
+    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) dst[j] = sm.ho[j];
+  }
   __device__ int tail_episode(Ctl &c) {
     int reason = R_NONE;
     Ctrl *x = p.ctrl;
@@ -1281,16 +1357,12 @@ struct Solver {
           for (int q = 0; q < 8; q++) x->ring[j][q] = 0;
       }
     }
-    grid_sync(&p.ctrl->bar, true);
-    nbar++;
-    if (p.trace && threadIdx.x == 0 && blockIdx.x == 0 && tn < p.trace_cap) {
-      p.trace[3 * tn] = 99; p.trace[3 * tn + 1] = reason; p.trace[3 * tn + 2] = (long long)gtime();
-      tn++;
-    }
-    reason = (int)ld_rlx((const u32 *)&x->ho_reason);
-    ph = (int)ld_rlx((const u32 *)&x->ho_ph) + 1;
-    long long *dst = reinterpret_cast<long long *>(&c);
-    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) dst[j] = ld_rlx(&x->ho[j]);
+    grid_sync(&p.ctrl->bar, true, [&] { load_handover(); });
+    if (lead()) L().nbar++;
+    trace_rec(99, reason);
+    reason = sm.ho_reason;
+    ph = sm.ho_ph + 1;
+    adopt_handover(c);
     return reason;
   }
 
@@ -1307,7 +1379,7 @@ struct Solver {
       int *Ac = Acp(c), *Ap = App(c);
       const int loop = (int)c.loop;
       bool act = false;
-      s_slots += c.len;
+      S(SS_SLOTS) += c.len;
       if (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) {  // SHRKRNL, slot order
         int out = 0;
         for (int i = 0; i < c.len; i++) {
@@ -1316,7 +1388,7 @@ struct Solver {
           if (a != -1) { st_rlx(p.iA + a, loop); act = true; Ac[out++] = a; }
         }
         c.len = out;
-        c.shrinks++;
+        if (lead()) L().shrinks++;
         c.shrink = 0;
       } else {  // INITKRNL (Alg. 8)
         for (int i = 0; i < c.len; i++) {
@@ -1339,7 +1411,7 @@ struct Solver {
           int x = ld_ro(p.cadj + j);
           u64 rs = ld_rlx(p.rowst + x);
           int l = labf(psi_of(rs), base, INF);
-          s_scan++;
+          S(SS_SCAN)++;
           if (l < psimin) {
             psimin = l; ub = x; wb = mu_of(rs);
             if (psimin == psiv - 1) break;
@@ -1350,7 +1422,7 @@ struct Solver {
       }
       c.ac0 ^= 1;
       c.loop++;
-      c.loops++;
+      if (lead()) L().loops++;
     }
   }
   __device__ int serial_episode(Ctl &c) {
@@ -1363,11 +1435,10 @@ struct Solver {
       const long long *src = reinterpret_cast<const long long *>(&c);
       for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) x->ho[j] = src[j];
     }
-    grid_sync(&p.ctrl->bar, false);
-    nbar++;
-    reason = (int)ld_rlx((const u32 *)&x->ho_reason);
-    long long *dst = reinterpret_cast<long long *>(&c);
-    for (int j = 0; j < (int)(sizeof(Ctl) / 8); j++) dst[j] = ld_rlx(&x->ho[j]);
+    grid_sync(&p.ctrl->bar, false, [&] { load_handover(); });
+    if (lead()) L().nbar++;
+    reason = sm.ho_reason;
+    adopt_handover(c);
     return reason;
   }
 
@@ -1397,10 +1468,10 @@ struct Solver {
       if (psimin < INF) {                                             // l.13-17
         st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));
         st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));
-        s_push++;
+        S(SS_PUSH)++;
       } else {                                                        // l.18-19
         st_rlx(p.colst + v, pack(-2, psi_of(cs)));
-        s_dead++;
+        S(SS_DEAD)++;
         atomicAdd(&p.ctrl->ndead, 1u);
       }
     }
@@ -1408,10 +1479,10 @@ struct Solver {
     add_count(act, 0);
     barrier<true>();
     const long long a = ring_prev(0);
-    c.ns_loop += (long long)(tnow() - l0);
+    if (lead()) L().ns_loop += (long long)(tnow() - l0);
     if (a == 0) return false;
     c.loop++;
-    c.loops++;
+    if (lead()) L().loops++;
     return true;
   }
 
@@ -1427,12 +1498,11 @@ struct Solver {
     int *U = Ub(c), *T = Tb(c);
     int ml = global_relabel<true>(U, c.ulen, T, Q4(0), Q4(1), c.base, Ac, gcount);
     c.u0 ^= 1;
-    c.grs++;
-    c.levels += ml / 2;
+    if (lead()) { L().grs++; L().levels += ml / 2; }
     c.base += stride();
-    c.ns_gr += (long long)(tnow() - g0);
+    if (lead()) L().ns_gr += (long long)(tnow() - g0);
     if (gcount == 0) return false;
-    c.guard_re += gcount;
+    if (lead()) L().guard_re += gcount;
     for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
       int v = __ldcg(Ac + i);
       u64 cs = ld_rlx(p.colst + v);
@@ -1440,7 +1510,7 @@ struct Solver {
       st_rlx(p.colst + v, pack(-1, psi_of(cs)));
       Ap[i] = v;
     }
-    barrier<true>();
+    barrier<true, false>();
     if (blockIdx.x == 0 && threadIdx.x == 0) p.ctrl->gcnt = 0;  // every CTA read it before the barrier above
     c.len = gcount;
     c.floor_r = c.floor_c = INF;
@@ -1451,19 +1521,20 @@ struct Solver {
   }
 
   // ---------------------------------------------------------------- the solve
-  __device__ void run() {
-    const bool lead = blockIdx.x == 0 && threadIdx.x == 0;
+  __device__ __forceinline__ void run() {
     u64 t0 = tnow(), tA = t0;
     long long ns_init = 0;
     int *Ac = p.wl0, *Ap = p.wl1;
     int *U = p.qa, *T = p.qb;
     int4 *Qa = Q4(0), *Qb = Q4(1);
-    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; }
+    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
+    for (int k = 0; k < SS_N; k++) sm.ts[k][threadIdx.x] = 0;
+    if (threadIdx.x < 2) sm.lvc[threadIdx.x] = 0;
     init_state();
-    barrier<true>();
+    barrier<true, false>();
     if (p.mode == MODE_SOLVE && p.init == 0) {
       greedy();
-      barrier<true>();
+      barrier<true, false>();
     }
     debug_check(1, -1, nullptr, 0);
     // unmatched rows -> U; unmatched columns (increasing id) -> Ac (R12)
@@ -1475,23 +1546,23 @@ struct Solver {
     int len = compact_pass2<true>(n, T, Ac, run1, Ap);  // Ap = Ac (R12)
     long long init_card = (long long)m - n_iso - ulen;
 
-    if (p.mode == MODE_GAP) {  // mcm_gap_relabel: labels in, labels out
+    if ((F & F_AUX) && p.mode == MODE_GAP) {  // mcm_gap_relabel: labels in, labels out
       int gl = gap_relabel(1);
       write_labels(1);
-      if (lead) p.ctrl->stat[ST_MAXLEVEL] = gl;
-      finish_stats(0, 0, 0, 0, 0, 0, 0, 0, 0, 0, 0);
+      if (lead()) p.ctrl->stat[ST_MAXLEVEL] = gl;
+      finish_stats(0, 0, 0);
       return;
     }
-    if (p.mode == MODE_RELABEL) {
+    if ((F & F_AUX) && p.mode == MODE_RELABEL) {
       int g;
       int ml = global_relabel<true>(U, ulen, T, Qa, Qb, 1, nullptr, g);
       write_labels(1);
-      if (lead) p.ctrl->stat[ST_MAXLEVEL] = ml;
-      finish_stats(0, 0, 0, 0, 0, 0, 0, 0, 0, 0, 0);
+      if (lead()) p.ctrl->stat[ST_MAXLEVEL] = ml;
+      finish_stats(0, 0, 0);
       return;
     }
 
-    barrier<true>();
+    barrier<true, false>();
     debug_check(2, -1, Ac, len);
     ns_init = (long long)(tnow() - t0);
 
@@ -1501,13 +1572,13 @@ struct Solver {
     c.floor_r = c.floor_c = INF;
     for (;;) {
       if (c.loop >= p.max_loops) {
-        if (lead) p.ctrl->err = -5;
+        if (lead()) p.ctrl->err = -5;
         break;
       }
-      if (p.serial && !c.gr_active && c.loop != c.iterGR && c.loop != c.gapAt) {
+      if ((F & F_SERIAL) && p.serial && !c.gr_active && c.loop != c.iterGR && c.loop != c.gapAt) {
         int r = serial_episode(c);
         if (r == R_CAP) {
-          if (lead) p.ctrl->err = -5;
+          if (lead()) p.ctrl->err = -5;
           break;
         }
         if (r == R_TERM && !guard_step(c)) break;
@@ -1522,7 +1593,7 @@ struct Solver {
       if (tail_ok) {
         int r = tail_episode(c);
         if (r == R_CAP) {
-          if (lead) p.ctrl->err = -5;
+          if (lead()) p.ctrl->err = -5;
           break;
         }
         if (r == R_TERM && !guard_step(c)) break;
@@ -1530,11 +1601,11 @@ struct Solver {
       }
       // one unit of grid work
       if (c.gr_active) { gr_step<true>(c); continue; }                // Alg. 5 level
-      if (c.loop == c.gapAt) {                                         // gap relabel (R14)
+      if ((F & F_GAP) && c.loop == c.gapAt) {                          // gap relabel (R14)
         u64 g0 = tnow();
-        if (gap_relabel(c.base - stride()) >= 0) c.gaps++;
+        if (gap_relabel(c.base - stride()) >= 0 && lead()) L().gaps++;
         c.gapAt = -1;
-        c.ns_gr += (long long)(tnow() - g0);
+        if (lead()) L().ns_gr += (long long)(tnow() - g0);
         continue;
       }
       if (c.loop == c.iterGR) {                                        // Alg. 7 l.6-9
@@ -1542,17 +1613,15 @@ struct Solver {
         gr_begin<true>(c);
         continue;
       }
-      if (p.variant == 1) {                                             // G-PR-First (Alg. 3)
+      if ((F & F_FIRST) && p.variant == 1) {                                             // G-PR-First (Alg. 3)
         if (!first_step(c) && !guard_step(c)) break;
         continue;
       }
       if (!loop_step<true>(c, Acp(c), App(c)) && !guard_step(c)) break;  // l.10-19 / termination
     }
-    gaps_total = c.gaps;
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
-    finish_stats(c.loops + c.tail_loops, c.grs, c.levels, c.shrinks, c.guard_re, init_card, ns_init, c.ns_gr,
-                 c.ns_loop, (long long)(tnow() - tA), c.tail_loops);
+    finish_stats(init_card, ns_init, (long long)(tnow() - tA));
   }
 
   __device__ void reset_labels() {
@@ -1562,30 +1631,29 @@ struct Solver {
       st_rlx(p.rowst + u, pack(mu_of(w), 0));
     }
     for (int v = g; v < n; v += G) { u64 w = ld_rlx(p.colst + v); st_rlx(p.colst + v, pack(mu_of(w), 0)); }
-    barrier<true>();
+    barrier<true, false>();
   }
 
-  __device__ void finish_stats(long long loops, long long grs, long long levels, long long shrinks, long long guard_re,
-                               long long init_card, long long ns_init, long long ns_gr, long long ns_loop,
-                               long long ns_total, long long tail_loops) {
-    long long v[10] = {s_push, s_block, s_dead, s_scan, s_slots, s_free, s_grrows, s_gredges, s_grcols, s_gyedges};
-    const int slot[10] = {ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_REACHED_FREE,
-                          ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES};
-    for (int k = 0; k < 10; k++) {
-      long long t = cta_sum<NT>(v[k], sm.red);
+  __device__ void finish_stats(long long init_card, long long ns_init, long long ns_total) {
+    __syncthreads();
+    const int slot[SS_N] = {ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_REACHED_FREE,
+                            ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES};
+    for (int k = 0; k < SS_N; k++) {
+      const long long t = cta_sum<NT>((long long)sm.ts[k][threadIdx.x], sm.red);
       if (threadIdx.x == 0 && t) atomicAdd((unsigned long long *)&p.ctrl->stat[slot[k]], (unsigned long long)t);
     }
-    if (blockIdx.x == 0 && threadIdx.x == 0) {
+    if (lead()) {
       long long *st = p.ctrl->stat;
-      st[ST_LOOPS] = loops; st[ST_GRS] = grs; st[ST_LEVELS] = levels; st[ST_SHRINKS] = shrinks;
-      st[ST_GAPS] = gaps_total;
-      st[ST_GUARD] = guard_re; st[ST_INITCARD] = init_card; st[ST_NS_INIT] = ns_init; st[ST_NS_GR] = ns_gr;
-      st[ST_NS_LOOP] = ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = tail_loops;
-      st[ST_BARRIERS] = nbar;
-      st[ST_TRACE_N] = tn;
+      const LeadStats &l = L();
+      st[ST_LOOPS] = l.loops + l.tail_loops; st[ST_GRS] = l.grs; st[ST_LEVELS] = l.levels; st[ST_SHRINKS] = l.shrinks;
+      st[ST_GAPS] = l.gaps;
+      st[ST_GUARD] = l.guard_re; st[ST_INITCARD] = init_card; st[ST_NS_INIT] = ns_init; st[ST_NS_GR] = l.ns_gr;
+      st[ST_NS_LOOP] = l.ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = l.tail_loops;
+      st[ST_BARRIERS] = l.nbar;
+      st[ST_TRACE_N] = l.tn;
       if (p.mode == MODE_SOLVE) {
-        st[ST_CARD] = (long long)ld_rlx(&p.ctrl->ring[(ph - 1) & 3][0]);
-        st[ST_FIXED] = (long long)ld_rlx(&p.ctrl->ring[(ph - 1) & 3][1]);
+        st[ST_CARD] = (long long)ring_prev(0);
+        st[ST_FIXED] = (long long)ring_prev(1);
       }
     }
   }
@@ -1594,8 +1662,9 @@ struct Solver {
 #ifndef MCM_MINB
 #define MCM_MINB 1
 #endif
+template <int F>
 __global__ void __launch_bounds__(NT, MCM_MINB) gpr_kernel(const __grid_constant__ Params p) {
-  Solver s(p);
+  Solver<F> s(p);
   s.run();
 }
 
