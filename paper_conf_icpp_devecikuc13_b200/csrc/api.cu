@@ -203,7 +203,7 @@ extern "C" {
 void mcm_default_options(mcm_options_t *o) {
   if (!o) return;
   memset(o, 0, sizeof(*o));
-  o->k = 0.7;
+  o->k = 0.4;  // the paper's best is 0.7; this build's measured best (R23)
   o->gr_strategy = MCM_GR_ADAPTIVE;
   o->shrink_min = 512;
   o->init = MCM_INIT_GREEDY;
@@ -386,10 +386,12 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
-  // the lean production instance unless a feature only the full one carries is on
-  void (*kern)(const Params) =
-      (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug) ? gpr_kernel<F_ALL> : gpr_kernel<F_FAST>;
   int C = o.tail_ctas;
+  // the lean production instance unless a feature only the full one carries is on
+  // (a cluster tail group spans several SMs' L1s: it needs gpu-scope vertex state)
+  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1)
+                                   ? gpr_kernel<F_ALL>
+                                   : gpr_kernel<F_FAST>;
   if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
   int maxg = h->max_grid;
   if (C > 1) {

@@ -55,6 +55,36 @@ __device__ __forceinline__ long long ld_rlx(const long long *p) {
   asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
   return v;
 }
+// Vertex-state accessors with a compile-time scope.  CTA scope may be served by
+// the SM's L1 (a dependent miss costs ~140 ns instead of 175-230 ns for the strong
+// gpu-scope load, a hit after this SM's own store ~30 ns instead of ~165 ns);
+// every grid barrier invalidates L1 (its __threadfence emits CCTL.IVALL), so a
+// phase always starts from L2's values and a racy read inside a phase may at
+// most be stale -- the paper's execution model (reading R17).
+template <bool CTA>
+__device__ __forceinline__ u64 ldv(const u64 *p) {
+  u64 v;
+  if (CTA) asm volatile("ld.relaxed.cta.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  else asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+template <bool CTA>
+__device__ __forceinline__ void stv(u64 *p, u64 v) {
+  if (CTA) asm volatile("st.relaxed.cta.global.b64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+  else asm volatile("st.relaxed.gpu.global.b64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+template <bool CTA>
+__device__ __forceinline__ int ldv(const int *p) {
+  int v;
+  if (CTA) asm volatile("ld.relaxed.cta.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  else asm volatile("ld.relaxed.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+  return v;
+}
+template <bool CTA>
+__device__ __forceinline__ void stv(int *p, int v) {
+  if (CTA) asm volatile("st.relaxed.cta.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+  else asm volatile("st.relaxed.gpu.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
 __device__ __forceinline__ u32 ld_acq(const u32 *p) {
   u32 v;
   asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");

@@ -137,13 +137,19 @@ __device__ __forceinline__ u64 tnow() { return (threadIdx.x == 0 && blockIdx.x =
 // (serial mode, G-PR-First, debug checks, gap relabelling, the label-only modes)
 // live in a second instance, so they cost the hot kernel no code size (its
 // instruction footprint is on the critical path of every short phase).
-enum { F_SERIAL = 1, F_FIRST = 2, F_DEBUG = 4, F_GAP = 8, F_AUX = 16, F_BU = 32 };
-constexpr int F_FAST = F_BU;
+enum { F_SERIAL = 1, F_FIRST = 2, F_DEBUG = 4, F_GAP = 8, F_AUX = 16, F_BU = 32, F_L1 = 64 };
+constexpr int F_FAST = F_BU | F_L1;  // F_L1: CTA-scope vertex state (single-CTA tail only)
 constexpr int F_ALL = F_SERIAL | F_FIRST | F_DEBUG | F_GAP | F_AUX | F_BU;
 
 template <int F>
 struct Solver {
   const Params &p;
+  // vertex state (rowst, colst, iA) scope: CTA (L1-cacheable) in the lean kernel
+  static constexpr bool VCTA = (F & F_L1) != 0;
+  __device__ __forceinline__ static u64 vld(const u64 *a) { return ldv<VCTA>(a); }
+  __device__ __forceinline__ static int vld(const int *a) { return ldv<VCTA>(a); }
+  __device__ __forceinline__ static void vst(u64 *a, u64 v) { stv<VCTA>(a, v); }
+  __device__ __forceinline__ static void vst(int *a, int v) { stv<VCTA>(a, v); }
   // the dynamic shared block, named through a namespace-scope extern __shared__
   // array so every access compiles to a shared-space instruction (a Smem& member
   // made the staging atomics generic ATOM.E)
@@ -241,10 +247,10 @@ struct Solver {
 
   __device__ __forceinline__ bool col_unmatched(int v) const {
     // R1: mu(v) = -1, or mu(v) >= 0 and mu(mu(v)) != v.  mu(v) = -2 (dead) is inactive.
-    int c = mu_of(ld_rlx(p.colst + v));
+    int c = mu_of(vld(p.colst + v));
     if (c == -1) return true;
     if (c < 0) return false;
-    return mu_of(ld_rlx(p.rowst + c)) != v;
+    return mu_of(vld(p.rowst + c)) != v;
   }
 
   // ---------------------------------------------------------------- staging
@@ -362,20 +368,20 @@ struct Solver {
     if (p.mode == MODE_GAP) {
       for (int u = g; u < m; u += G) {
         int l = p.rmatch_in[u];
-        st_rlx(p.rowst + u, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
+        vst(p.rowst + u, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
       }
       for (int v = g; v < n; v += G) {
         int l = p.cmatch_in[v];
-        st_rlx(p.colst + v, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
+        vst(p.colst + v, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
       }
       return;
     }
     const bool given = (p.mode == MODE_RELABEL) || (p.init == 1);
     for (int u = g; u < m; u += G) {
-      st_rlx(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
+      vst(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
     }
     for (int v = g; v < n; v += G) {
-      st_rlx(p.colst + v, pack(given ? p.cmatch_in[v] : -1, 0));
+      vst(p.colst + v, pack(given ? p.cmatch_in[v] : -1, 0));
       p.iA[v] = -1;  // R12
     }
   }
@@ -399,14 +405,14 @@ struct Solver {
 #pragma unroll
           for (int k = 0; k < KB; k++) u[k] = j0 + k < e ? ld_ro(p.cadj + j0 + k) : -1;
 #pragma unroll
-          for (int k = 0; k < KB; k++) rs[k] = u[k] >= 0 ? ld_rlx(p.rowst + u[k]) : 0ull;
+          for (int k = 0; k < KB; k++) rs[k] = u[k] >= 0 ? vld(p.rowst + u[k]) : 0ull;
 #pragma unroll
           for (int k = 0; k < KB; k++) {
             if (done || u[k] < 0) continue;
             S(SS_GYEDGES)++;
             if (mu_of(rs[k]) != -1) continue;
             if (atomicCAS(p.rowst + u[k], rs[k], pack(v, psi_of(rs[k]))) == rs[k]) {
-              st_rlx(p.colst + v, pack(u[k], 0));
+              vst(p.colst + v, pack(u[k], 0));
               done = true;
             }
           }
@@ -423,7 +429,7 @@ struct Solver {
           int j = c0 + lane;
           int u = -1;
           u64 rs = 0;
-          if (j < eb) { u = ld_ro(p.cadj + j); rs = ld_rlx(p.rowst + u); S(SS_GYEDGES)++; }
+          if (j < eb) { u = ld_ro(p.cadj + j); rs = vld(p.rowst + u); S(SS_GYEDGES)++; }
           unsigned cand = __ballot_sync(0xffffffffu, u >= 0 && mu_of(rs) == -1);
           while (cand && !done) {
             int l = __ffs(cand) - 1;
@@ -431,7 +437,7 @@ struct Solver {
             int ok = 0;
             if (lane == l) {
               ok = atomicCAS(p.rowst + u, rs, pack(vb, psi_of(rs))) == rs;
-              if (ok) st_rlx(p.colst + vb, pack(u, 0));
+              if (ok) vst(p.colst + vb, pack(u, 0));
             }
             done = __shfl_sync(0xffffffffu, ok, l);
           }
@@ -447,7 +453,7 @@ struct Solver {
     long long iso = 0;
     for (int t = blockIdx.x * NT; t < m; t += gridDim.x * NT) {
       int u = t + threadIdx.x;
-      bool f = u < m && mu_of(ld_rlx(p.rowst + u)) == -1;
+      bool f = u < m && mu_of(vld(p.rowst + u)) == -1;
       if (f && p.mode == MODE_SOLVE && ld_ro(p.rptr + u) == ld_ro(p.rptr + u + 1)) { f = false; iso++; }
       int tot, r = cta_rank<NT>(f, sm.w, &tot);
       if (threadIdx.x == 0) sm.qbase = tot ? (int)atomicAdd(ring_now(j), (u32)tot) : 0;
@@ -496,8 +502,8 @@ struct Solver {
         u = (i < curlen) ? ld_cg(cur0 + i) : -1;
         bool keep = false;
         if (u >= 0) {
-          if (mu_of(ld_rlx(p.rowst + u)) == -1) {
-            if (gl == 0) st_rlx(p.rowst + u, pack(-1, base));
+          if (mu_of(vld(p.rowst + u)) == -1) {
+            if (gl == 0) vst(p.rowst + u, pack(-1, base));
             keep = gl == 0;
           } else {
             u = -1;
@@ -545,7 +551,7 @@ struct Solver {
         v[k] = jj < e ? ld_ro(p.radj + jj) : -1;
       }
 #pragma unroll
-      for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? ld_rlx(p.colst + v[k]) : ~0ull;
+      for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : ~0ull;
       if (spec) {  // narrow level: mate loads ride along with the CAS (one round trip)
 #pragma unroll
         for (int k = 0; k < KB; k++) {
@@ -554,7 +560,7 @@ struct Solver {
           const int w = mu_of(cs[k]);
           old[k] = try_ ? atomicCAS(p.colst + v[k], cs[k], pack(w, lc)) : ~cs[k];
           const bool go = try_ && w >= 0;
-          rw[k] = go ? ld_rlx(p.rowst + w) : 0ull;
+          rw[k] = go ? vld(p.rowst + w) : 0ull;
           rs[k] = go ? ld_ro(p.rptr + w) : 0;
           re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
         }
@@ -568,7 +574,7 @@ struct Solver {
         for (int k = 0; k < KB; k++) {
           const int w = mu_of(cs[k]);
           const bool go = old[k] == cs[k] && w >= 0;
-          rw[k] = go ? ld_rlx(p.rowst + w) : 0ull;
+          rw[k] = go ? vld(p.rowst + w) : 0ull;
           rs[k] = go ? ld_ro(p.rptr + w) : 0;
           re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
         }
@@ -579,7 +585,7 @@ struct Solver {
         S(SS_GRCOLS)++;
         int w = mu_of(cs[k]);
         if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: mu(v) > -1 and mu(mu(v)) = v
-          st_rlx(p.rowst + w, pack(v[k], lr));
+          vst(p.rowst + w, pack(v[k], lr));
           stage(make_int4(w, rs[k], re[k], 0), next, ncnt);
         } else {
           S(SS_FREE)++;
@@ -607,7 +613,7 @@ struct Solver {
       int s = 0, e = 0;
       bool open = false, hit = false;
       if (v < n) {
-        cs = ld_rlx(p.colst + v);
+        cs = vld(p.colst + v);
         if (psi_of(cs) < base) {
           open = true;
           s = ld_ro(p.cptr + v);
@@ -621,7 +627,7 @@ struct Solver {
 #pragma unroll
           for (int k = 0; k < KB; k++) x[k] = j + k < e ? ld_ro(p.cadj + j + k) : -1;
 #pragma unroll
-          for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+          for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
 #pragma unroll
           for (int k = 0; k < KB; k++) hit |= x[k] >= 0 && psi_of(rs[k]) == lf;
           S(SS_GREDGES) += min(KB, e - j);
@@ -638,7 +644,7 @@ struct Solver {
 #pragma unroll
           for (int k = 0; k < KB; k++) {
             const int jj = c0 + k * 32 + lane;
-            if (jj < eb) h |= psi_of(ld_rlx(p.rowst + ld_ro(p.cadj + jj))) == lf;
+            if (jj < eb) h |= psi_of(vld(p.rowst + ld_ro(p.cadj + jj))) == lf;
           }
           any = __any_sync(0xffffffffu, h);
           if (lane == 0) S(SS_GREDGES) += min(32 * KB, eb - c0);
@@ -646,14 +652,14 @@ struct Solver {
         if (lane == bl) hit = any;
       }
       if (hit) {
-        st_rlx(p.colst + v, pack(mu_of(cs), lc));
+        vst(p.colst + v, pack(mu_of(cs), lc));
         S(SS_GRCOLS)++;
         const int w = mu_of(cs);
         u64 rw = 0;
         int rs = 0, re = 0;
-        if (w >= 0) { rw = ld_rlx(p.rowst + w); rs = ld_ro(p.rptr + w); re = ld_ro(p.rptr + w + 1); }
+        if (w >= 0) { rw = vld(p.rowst + w); rs = ld_ro(p.rptr + w); re = ld_ro(p.rptr + w + 1); }
         if (w >= 0 && mu_of(rw) == v) {  // matched: its mate joins the next level
-          st_rlx(p.rowst + w, pack(v, lr));
+          vst(p.rowst + w, pack(v, lr));
           stage(make_int4(w, rs, re, 0), next, ncnt);
         } else {
           S(SS_FREE)++;
@@ -763,7 +769,7 @@ struct Solver {
     } else {
       a = ld_wl(Ac + i);
     }
-    if (a != -1) st_rlx(p.iA + a, loop);
+    if (a != -1) vst(p.iA + a, loop);
     return a;
   }
 
@@ -789,9 +795,9 @@ struct Solver {
     // (dead columns are counted for the early-stop GR target, R22)
     int psimin = best == ~0ull ? INF : (int)(best >> 32);
     if (psimin < INF) {                                 // l.12
-      if (wb == -1 || ld_rlx(p.iA + wb) != loop) {      // l.13
-        st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
-        st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
+      if (wb == -1 || vld(p.iA + wb) != loop) {      // l.13
+        vst(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
+        vst(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
         Ap[i] = wb;                                     // l.18 (R3)
         S(SS_PUSH)++;
       } else {
@@ -799,7 +805,7 @@ struct Solver {
         S(SS_BLOCK)++;
       }
     } else {
-      st_rlx(p.colst + v, pack(-2, psi_of(cs)));        // l.20
+      vst(p.colst + v, pack(-2, psi_of(cs)));        // l.20
       Ac[i] = -1;                                       // l.21
       Ap[i] = -1;                                       // l.22
       S(SS_DEAD)++;
@@ -819,7 +825,7 @@ struct Solver {
       int s = 0, e = 0, psiv = INF;
       u64 cs = 0;
       if (v >= 0) {
-        cs = ld_rlx(p.colst + v);
+        cs = vld(p.colst + v);
         psiv = labf(psi_of(cs), base, fl_c);
         s = ld_ro(p.cptr + v);
         e = ld_ro(p.cptr + v + 1);
@@ -893,7 +899,7 @@ struct Solver {
         x[k] = jj < e ? ld_ro(p.cadj + jj) : -1;
       }
 #pragma unroll
-      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
       u64 key = ~0ull;
       int kx = -1, kw = -1;
 #pragma unroll
@@ -951,7 +957,7 @@ struct Solver {
         x[k] = jj < e ? ld_ro(p.cadj + s + q) : -1;
       }
 #pragma unroll
-      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? ld_rlx(p.rowst + x[k]) : 0ull;
+      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
       u64 key = ~0ull;
       int kx = -1, kw = -1;
 #pragma unroll
@@ -984,13 +990,13 @@ struct Solver {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     long long card = 0, fixed = 0;
     for (int u = g; u < m; u += G) {
-      int c = mu_of(ld_rlx(p.rowst + u));
+      int c = mu_of(vld(p.rowst + u));
       p.rmatch_out[u] = c;
       card += c >= 0;
     }
     for (int v = g; v < n; v += G) {
-      int c = mu_of(ld_rlx(p.colst + v));
-      int ok = (c >= 0 && mu_of(ld_rlx(p.rowst + c)) == v) ? c : -1;
+      int c = mu_of(vld(p.colst + v));
+      int ok = (c >= 0 && mu_of(vld(p.rowst + c)) == v) ? c : -1;
       fixed += (c != -1 && ok == -1);
       p.cmatch_out[v] = ok;
     }
@@ -1000,8 +1006,8 @@ struct Solver {
 
   __device__ void write_labels(u32 base) {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
-    for (int u = g; u < m; u += G) p.rmatch_out[u] = lab(psi_of(ld_rlx(p.rowst + u)), base, INF);
-    for (int v = g; v < n; v += G) p.cmatch_out[v] = lab(psi_of(ld_rlx(p.colst + v)), base, INF);
+    for (int u = g; u < m; u += G) p.rmatch_out[u] = lab(psi_of(vld(p.rowst + u)), base, INF);
+    for (int v = g; v < n; v += G) p.cmatch_out[v] = lab(psi_of(vld(p.colst + v)), base, INF);
   }
 
   __device__ int iter_gap(int maxLevel) const {
@@ -1021,8 +1027,8 @@ struct Solver {
     if (!(F & F_DEBUG) || !p.debug) return;
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     for (int u = g; u < m; u += G) {
-      int c = mu_of(ld_rlx(p.rowst + u));
-      if (c >= 0 && mu_of(ld_rlx(p.colst + c)) != u) dbg_record(where, loop, u, c);
+      int c = mu_of(vld(p.rowst + u));
+      if (c >= 0 && mu_of(vld(p.colst + c)) != u) dbg_record(where, loop, u, c);
     }
     for (int v = g; v < n; v += G) p.dbgbuf[v] = 0;
     barrier<true, false>();
@@ -1056,7 +1062,7 @@ struct Solver {
     __syncthreads();
     int lmax = -1;
     for (int x = g; x < m + n; x += G) {
-      u64 w = ld_rlx(x < m ? p.rowst + x : p.colst + (x - m));
+      u64 w = vld(x < m ? p.rowst + x : p.colst + (x - m));
       int l = lab(psi_of(w), base, INF);
       if (l < INF) {
         if (l < SH) atomicAdd(&sm.q[l], 1);
@@ -1085,9 +1091,9 @@ struct Solver {
     if (gap != 0x7fffffff) {
       for (int x = g; x < m + n; x += G) {
         u64 *a = x < m ? p.rowst + x : p.colst + (x - m);
-        u64 w = ld_rlx(a);
+        u64 w = vld(a);
         int l = lab(psi_of(w), base, INF);
-        if (l > gap && l < INF) { st_rlx(a, pack(mu_of(w), 0)); killed++; }  // psi 0 < base: infinite
+        if (l > gap && l < INF) { vst(a, pack(mu_of(w), 0)); killed++; }  // psi 0 < base: infinite
       }
     }
     for (int l = g; l < L; l += G) p.hist[l] = 0;
@@ -1385,7 +1391,7 @@ struct Solver {
         for (int i = 0; i < c.len; i++) {
           int v = Ap[i], a = Ac[i];
           if (v != -1 && col_unmatched(v)) a = v;
-          if (a != -1) { st_rlx(p.iA + a, loop); act = true; Ac[out++] = a; }
+          if (a != -1) { vst(p.iA + a, loop); act = true; Ac[out++] = a; }
         }
         c.len = out;
         if (lead()) L().shrinks++;
@@ -1395,21 +1401,21 @@ struct Solver {
           int v = Ap[i];
           if (v != -1 && col_unmatched(v)) Ac[i] = v;
           v = Ac[i];
-          if (v != -1) { st_rlx(p.iA + v, loop); act = true; }
+          if (v != -1) { vst(p.iA + v, loop); act = true; }
         }
       }
       if (!act) { reason = R_TERM; return; }
       for (int i = 0; i < c.len; i++) {  // PUSHKRNL (Alg. 9)
         int v = Ac[i];
         if (v == -1) { Ap[i] = -1; continue; }
-        u64 cs = ld_rlx(p.colst + v);
+        u64 cs = vld(p.colst + v);
         int psiv = labf(psi_of(cs), base, INF);
         int s = ld_ro(p.cptr + v), e = ld_ro(p.cptr + v + 1);
         if (p.dead_skip && psiv >= INF) e = s;
         int psimin = INF, ub = -1, wb = -1;
         for (int j = s; j < e; j++) {
           int x = ld_ro(p.cadj + j);
-          u64 rs = ld_rlx(p.rowst + x);
+          u64 rs = vld(p.rowst + x);
           int l = labf(psi_of(rs), base, INF);
           S(SS_SCAN)++;
           if (l < psimin) {
@@ -1453,9 +1459,9 @@ struct Solver {
     fl_r = c.floor_r;
     fl_c = c.floor_c;
     for (int v = g; v < n; v += G) {
-      u64 cs = ld_rlx(p.colst + v);
+      u64 cs = vld(p.colst + v);
       int cm = mu_of(cs);
-      bool active = cm == -1 || (cm >= 0 && mu_of(ld_rlx(p.rowst + cm)) != v);  // Alg. 6 l.3 (R1)
+      bool active = cm == -1 || (cm >= 0 && mu_of(vld(p.rowst + cm)) != v);  // Alg. 6 l.3 (R1)
       if (!active) continue;
       act++;
       int psiv = labf(psi_of(cs), base, fl_c);
@@ -1466,11 +1472,11 @@ struct Solver {
       scan(s, e, 0, 1, 1u << lane_id(), psiv - 1, base, best, ub, wb);  // l.5-12
       int psimin = best == ~0ull ? INF : (int)(best >> 32);
       if (psimin < INF) {                                             // l.13-17
-        st_rlx(p.rowst + ub, pack(v, base + (u32)psimin + 2u));
-        st_rlx(p.colst + v, pack(ub, base + (u32)psimin + 1u));
+        vst(p.rowst + ub, pack(v, base + (u32)psimin + 2u));
+        vst(p.colst + v, pack(ub, base + (u32)psimin + 1u));
         S(SS_PUSH)++;
       } else {                                                        // l.18-19
-        st_rlx(p.colst + v, pack(-2, psi_of(cs)));
+        vst(p.colst + v, pack(-2, psi_of(cs)));
         S(SS_DEAD)++;
         atomicAdd(&p.ctrl->ndead, 1u);
       }
@@ -1505,9 +1511,9 @@ struct Solver {
     if (lead()) L().guard_re += gcount;
     for (int i = blockIdx.x * NT + threadIdx.x; i < gcount; i += gridDim.x * NT) {
       int v = __ldcg(Ac + i);
-      u64 cs = ld_rlx(p.colst + v);
+      u64 cs = vld(p.colst + v);
       if (mu_of(cs) == -2) atomicSub(&p.ctrl->ndead, 1u);
-      st_rlx(p.colst + v, pack(-1, psi_of(cs)));
+      vst(p.colst + v, pack(-1, psi_of(cs)));
       Ap[i] = v;
     }
     barrier<true, false>();
@@ -1627,10 +1633,10 @@ struct Solver {
   __device__ void reset_labels() {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     for (int u = g; u < m; u += G) {
-      u64 w = ld_rlx(p.rowst + u);
-      st_rlx(p.rowst + u, pack(mu_of(w), 0));
+      u64 w = vld(p.rowst + u);
+      vst(p.rowst + u, pack(mu_of(w), 0));
     }
-    for (int v = g; v < n; v += G) { u64 w = ld_rlx(p.colst + v); st_rlx(p.colst + v, pack(mu_of(w), 0)); }
+    for (int v = g; v < n; v += G) { u64 w = vld(p.colst + v); vst(p.colst + v, pack(mu_of(w), 0)); }
     barrier<true, false>();
   }
 

@@ -39,7 +39,7 @@ def test_host_only_calls():
     import paper_conf_icpp_devecikuc13_b200 as pkg
 
     o = pkg.mcm_default_options()
-    assert o.k == 0.7 and o.shrink_min == 512 and o.gr_strategy == 0 and o.init == 0 and o.final_check == 1
+    assert o.k == 0.4 and o.shrink_min == 512 and o.gr_strategy == 0 and o.init == 0 and o.final_check == 1
     assert pkg.mcm_workspace_bytes(10, 10, 20) > 0
     assert pkg.mcm_workspace_bytes(-1, 10, 20) == 0
     assert pkg.mcm_workspace_bytes(1 << 30, 1 << 30, 5) == 0  # m+n+2 >= 2^31
