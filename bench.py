@@ -300,8 +300,8 @@ def run_ours(args, rank, world, local_rank):
             "algorithmic_bytes_per_launch": alg,
             "peak_source": "MEASURED_PEAKS.json hbm_gbs" if peaks else "fallback B200_PROFILING.md",
             "latency": {"grid_barriers": stats["grid_barriers"], "loops": stats["loops"],
-                        "gr_levels": stats["gr_levels"], "us_per_grid_barrier_measured": 1.21,
-                        "barrier_floor_ms": stats["grid_barriers"] * 1.21e-3},
+                        "gr_levels": stats["gr_levels"], "us_per_grid_barrier_measured": 1.27,
+                        "barrier_floor_ms": stats["grid_barriers"] * 1.27e-3},
         },
         "solve_stats": {k: stats[k] for k in ("loops", "gr_count", "gr_levels", "pushes", "blocked", "dead",
                                               "edges_scanned", "slots", "shrinks", "guard_reactivated",
