@@ -44,7 +44,10 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   L.iA = take(sizeof(int) * (size_t)n);
   L.wl0 = take(sizeof(int) * (size_t)n);
   L.wl1 = take(sizeof(int) * (size_t)n);
-  for (int i = 0; i < 4; i++) L.q[i] = take((i < 2 ? sizeof(int) : sizeof(int4)) * mx);  // q2, q3: int4 frontiers
+  // q2, q3: int4 BFS frontiers -- every row at most once per GR, plus the extra
+  // ranges of rows whose adjacency is split (stage_row)
+  for (int i = 0; i < 4; i++)
+    L.q[i] = take(i < 2 ? sizeof(int) * mx : sizeof(int4) * (mx + (size_t)nnz / SPLIT + 1));
   L.ctacnt = take(sizeof(int) * MAX_CTAS);
   L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
   L.hist_len = (int)std::min<long long>((long long)m + n + 2, 1 << 20);

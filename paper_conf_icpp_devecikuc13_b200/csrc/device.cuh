@@ -175,4 +175,30 @@ __device__ __forceinline__ int cta_rank(bool flag, int *s_w, int *total) {
   return off + r;
 }
 
+// Stable CTA-wide exclusive scan of a per-thread count (thread order); *total =
+// the CTA's sum.
+template <int NT>
+__device__ __forceinline__ int cta_scan(int x, int *s_w, int *total) {
+  constexpr int NW = NT / 32;
+  const int lane = lane_id(), w = warp_id();
+  int inc = x;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    int y = __shfl_up_sync(0xffffffffu, inc, o);
+    if (lane >= o) inc += y;
+  }
+  __syncthreads();
+  if (lane == 31) s_w[w] = inc;
+  __syncthreads();
+  int off = 0, tot = 0;
+#pragma unroll
+  for (int i = 0; i < NW; i++) {
+    int c = s_w[i];
+    off += (i < w) ? c : 0;
+    tot += c;
+  }
+  *total = tot;
+  return off + inc - x;
+}
+
 }  // namespace mcm

@@ -32,8 +32,10 @@ constexpr int SMALL_DEG = 32;    // greedy: adjacency lists up to this length: o
 constexpr int BIG_DEG = 64;      // GR / push: longer lists go to the whole warp
 constexpr int HUGE_DEG = 512;    // push: longer lists go to the whole CTA
 constexpr int MAXHUGE = 32;      // CTA-wide push list per tile
-constexpr int HUGE_CTA = 4;      // at most this many per tile: one CTA-wide scan each; more: a warp each
+constexpr int HUGE_CTA = 4;      // at most this many per tile: one CTA-wide scan each; more: a warp each ...
+constexpr int HUGE_WARP = 8192;  // ... unless longer than this
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
+constexpr int SPLIT = 1024;      // GR: a frontier row's adjacency is split into ranges of at most this many
 
 enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
 
@@ -117,6 +119,7 @@ struct Smem {
   u64 hugec[MAXHUGE];
   int huget[MAXHUGE];
   int nhuge;
+  u32 nd;                  // push: columns declared dead in this tile (-> Ctrl::ndead)
   int qcnt, qbase, tmp;
 };
 
@@ -253,6 +256,33 @@ struct Solver {
     return mu_of(vld(p.rowst + c)) != v;
   }
 
+  // R1 for columns i0 .. i0+RB-1 (< hi): val[k] = the column if unmatched, else -1.
+  // skip_iso: columns without any edge are left out as well (returns their count):
+  // they can never be matched, and a first push would only declare them dead
+  template <int RB>
+  __device__ __forceinline__ int cols_unmatched(int i0, int hi, int *val, bool skip_iso) const {
+    u64 cw[RB], rw[RB];
+    int cs[RB], ce[RB];
+#pragma unroll
+    for (int k = 0; k < RB; k++) cw[k] = i0 + k < hi ? vld(p.colst + i0 + k) : pack(-2, 0);
+#pragma unroll
+    for (int k = 0; k < RB; k++) rw[k] = mu_of(cw[k]) >= 0 ? vld(p.rowst + mu_of(cw[k])) : 0ull;
+#pragma unroll
+    for (int k = 0; k < RB; k++) {
+      const bool f = skip_iso && mu_of(cw[k]) == -1;
+      cs[k] = f ? ld_ro(p.cptr + i0 + k) : 0;
+      ce[k] = f ? ld_ro(p.cptr + i0 + k + 1) : 1;
+    }
+    int iso = 0;
+#pragma unroll
+    for (int k = 0; k < RB; k++) {
+      const int c = mu_of(cw[k]);
+      val[k] = (c == -1 || (c >= 0 && mu_of(rw[k]) != i0 + k)) ? i0 + k : -1;
+      if (c == -1 && cs[k] == ce[k]) { val[k] = -1; iso++; }
+    }
+    return iso;
+  }
+
   // ---------------------------------------------------------------- staging
   // BFS frontier entries are {row, rptr[row], rptr[row+1], 0}: the producer loads
   // the adjacency bounds of a row it discovers in parallel with its mate check, so
@@ -274,6 +304,28 @@ struct Solver {
       if (o.thread_rank() == 0) gb = atomicAdd(gcnt, (u32)o.size());
       gb = o.shfl(gb, 0);
       next[gb + o.thread_rank()] = x;
+    }
+  }
+  // A row joins the next frontier as the edge range [s, e) of its adjacency; a
+  // long list is split into ranges of SPLIT entries (w = 1 marks a continuation),
+  // each expanded independently at the next level -- an R-MAT hub row (1.5 * 10^5
+  // entries) on one warp held every level it appeared in for ~1.2 ms
+  __device__ __forceinline__ void stage_row(int w, int s, int e, int4 *next, u32 *gcnt) {
+    if (e - s <= SPLIT) {
+      stage(make_int4(w, s, e, 0), next, gcnt);
+      return;
+    }
+    for (int c = s; c < e; c += SPLIT) stage(make_int4(w, c, min(e, c + SPLIT), c > s), next, gcnt);
+  }
+  // one more alive unmatched column labelled by this GR (ring counter 2): warp-
+  // aggregated into a per-CTA shared counter that flush() publishes once per tile
+  // (one global atomic per reached column put ~10^6 same-address atomics on one
+  // L2 line in the first GRs of C3 / C4)
+  __device__ __forceinline__ void count_free() {
+    cg::coalesced_group g = cg::coalesced_threads();
+    if (g.thread_rank() == 0) {
+      if (sq) atomicAdd(ring_now(2), (u32)g.size());
+      else atomicAdd(&sm.lvc[0], (u32)g.size());
     }
   }
   __device__ __forceinline__ void flush(int4 *next, u32 *gcnt) {
@@ -302,6 +354,10 @@ struct Solver {
     __syncthreads();
     if (threadIdx.x == 0) {
       sm.qcnt = 0;
+      if (sm.lvc[0]) {
+        atomicAdd(ring_now(2), sm.lvc[0]);
+        sm.lvc[0] = 0;
+      }
       if (fe_on && sm.lvc[1]) {
         atomicAdd(ring_now(4), sm.lvc[1]);
         sm.lvc[1] = 0;
@@ -311,22 +367,29 @@ struct Solver {
   }
 
   // ---------------------------------------------------------------- stable compaction
-  // Pass 1 of a stable compaction of items [0, len): f(i) returns the value to keep
-  // or -1.  Survivors of CTA c's chunk go to T[lo_c + rank]; ctacnt[c] = count.
-  // GRID=false: a single CTA, written straight to `out` (reads of a tile finish
-  // before its writes, and writes never pass the tile being read).
-  template <bool GRID, class Fn>
+  // Pass 1 of a stable compaction of items [0, len): f(i0, hi, val) fills val[k]
+  // with the value to keep for item i0 + k (< hi) or -1 -- RB consecutive items per
+  // thread, so f can issue each stage's loads for all of them at once.  Survivors
+  // of CTA c's chunk go to T[lo_c + rank]; ctacnt[c] = count.  GRID=false: a single
+  // CTA, written straight to `out` (a tile's reads finish before its writes -- the
+  // scan's barrier separates them -- and writes never pass the tile being read).
+  template <bool GRID, int RB, class Fn>
   __device__ int compact_pass1(int len, Fn f, int *T, int *out) {
     const int C = ncta<GRID>(), c = cta<GRID>();
     const int chunk = (len + C - 1) / C;
     const int lo = min(len, c * chunk), hi = min(len, lo + chunk);
     int run = 0;
-    for (int t = lo; t < hi; t += NT) {
-      int i = t + threadIdx.x;
-      int val = (i < hi) ? f(i) : -1;
-      int tot;
-      int r = cta_rank<NT>(val != -1, sm.w, &tot);
-      if (val != -1) (C > 1 ? T[lo + run + r] : out[run + r]) = val;
+    for (int t = lo; t < hi; t += NT * RB) {
+      int val[RB];
+      f(t + (int)threadIdx.x * RB, hi, val);
+      int cnt = 0;
+#pragma unroll
+      for (int k = 0; k < RB; k++) cnt += val[k] != -1;
+      int tot, r = cta_scan<NT>(cnt, sm.w, &tot);
+      int *dst = (C > 1 ? T + lo : out) + run + r;
+#pragma unroll
+      for (int k = 0; k < RB; k++)
+        if (val[k] != -1) *dst++ = val[k];
       run += tot;
     }
     if (C > 1 && threadIdx.x == 0) p.ctacnt[c] = run;
@@ -391,55 +454,110 @@ struct Solver {
   // neighbour is taken, so the result is maximal.  (Outside the push loop, the
   // paper's atomic-free claim concerns the push-relabel steps.)
   __device__ void greedy() {
+    // RG columns per lane (a warp tile of 32*RG columns): the bounds, the first KB
+    // candidates and their row words of all RG columns are loaded stage by stage and
+    // the RG claims issued together, so a thread keeps RG independent chains in
+    // flight; a column whose first free candidate was taken meanwhile (or that has
+    // none among its first KB) continues alone from there.
+    constexpr int RG = 4;
     const int lane = lane_id();
     const int gw = (blockIdx.x * NT + threadIdx.x) >> 5, NWG = gridDim.x * NWARP;
-    for (int b = gw * 32; b < n; b += NWG * 32) {
-      int v = b + lane;
-      int s = 0, e = 0;
-      if (v < n) { s = ld_ro(p.cptr + v); e = ld_ro(p.cptr + v + 1); }
-      if (v < n && e - s <= SMALL_DEG) {
-        bool done = false;
-        for (int j0 = s; j0 < e && !done; j0 += KB) {  // KB candidates in flight
-          int u[KB];
-          u64 rs[KB];
+    for (long long b = (long long)gw * 32 * RG; b < n; b += (long long)NWG * 32 * RG) {
+      int v[RG], s[RG], e[RG];
 #pragma unroll
-          for (int k = 0; k < KB; k++) u[k] = j0 + k < e ? ld_ro(p.cadj + j0 + k) : -1;
+      for (int k = 0; k < RG; k++) {
+        const long long x = b + k * 32 + lane;
+        v[k] = x < n ? (int)x : -1;
+      }
 #pragma unroll
-          for (int k = 0; k < KB; k++) rs[k] = u[k] >= 0 ? vld(p.rowst + u[k]) : 0ull;
+      for (int k = 0; k < RG; k++) {
+        s[k] = v[k] >= 0 ? ld_ro(p.cptr + v[k]) : 0;
+        e[k] = v[k] >= 0 ? ld_ro(p.cptr + v[k] + 1) : 0;
+      }
+      int u[RG][KB];
+      u64 rs[RG][KB];
 #pragma unroll
-          for (int k = 0; k < KB; k++) {
-            if (done || u[k] < 0) continue;
-            S(SS_GYEDGES)++;
-            if (mu_of(rs[k]) != -1) continue;
-            if (atomicCAS(p.rowst + u[k], rs[k], pack(v, psi_of(rs[k]))) == rs[k]) {
-              vst(p.colst + v, pack(u[k], 0));
-              done = true;
+      for (int k = 0; k < RG; k++)
+#pragma unroll
+        for (int q = 0; q < KB; q++)
+          u[k][q] = s[k] + q < e[k] ? ld_ro(p.cadj + s[k] + q) : -1;
+#pragma unroll
+      for (int k = 0; k < RG; k++)
+#pragma unroll
+        for (int q = 0; q < KB; q++) rs[k][q] = u[k][q] >= 0 ? vld(p.rowst + u[k][q]) : 0ull;
+      int pos[RG];
+      bool done[RG];
+      u64 exp_[RG], old[RG];
+      int cu[RG];
+#pragma unroll
+      for (int k = 0; k < RG; k++) {
+        int pick = -1;
+#pragma unroll
+        for (int q = KB - 1; q >= 0; q--)
+          if (u[k][q] >= 0 && mu_of(rs[k][q]) == -1) pick = q;
+        const int deg = e[k] - s[k];
+        if (v[k] >= 0) S(SS_GYEDGES) += pick >= 0 ? pick + 1 : min(deg, KB);
+        cu[k] = -1;
+        exp_[k] = 0;
+#pragma unroll
+        for (int q = 0; q < KB; q++)
+          if (q == pick) { cu[k] = u[k][q]; exp_[k] = rs[k][q]; }
+        pos[k] = pick >= 0 ? s[k] + pick + 1 : s[k] + KB;
+      }
+#pragma unroll
+      for (int k = 0; k < RG; k++)
+        old[k] = cu[k] >= 0 ? atomicCAS(p.rowst + cu[k], exp_[k], pack(v[k], psi_of(exp_[k]))) : ~exp_[k];
+#pragma unroll
+      for (int k = 0; k < RG; k++) {
+        done[k] = cu[k] >= 0 && old[k] == exp_[k];
+        if (done[k]) vst(p.colst + v[k], pack(cu[k], 0));
+      }
+#pragma unroll
+      for (int k = 0; k < RG; k++) {
+        if (v[k] >= 0 && e[k] - s[k] <= SMALL_DEG && !done[k]) {  // the rest of a short list, alone
+          bool dn = false;
+          for (int j0 = pos[k]; j0 < e[k] && !dn; j0 += KB) {
+            int uu[KB];
+            u64 rr[KB];
+#pragma unroll
+            for (int q = 0; q < KB; q++) uu[q] = j0 + q < e[k] ? ld_ro(p.cadj + j0 + q) : -1;
+#pragma unroll
+            for (int q = 0; q < KB; q++) rr[q] = uu[q] >= 0 ? vld(p.rowst + uu[q]) : 0ull;
+#pragma unroll
+            for (int q = 0; q < KB; q++) {
+              if (dn || uu[q] < 0) continue;
+              S(SS_GYEDGES)++;
+              if (mu_of(rr[q]) != -1) continue;
+              if (atomicCAS(p.rowst + uu[q], rr[q], pack(v[k], psi_of(rr[q]))) == rr[q]) {
+                vst(p.colst + v[k], pack(uu[q], 0));
+                dn = true;
+              }
             }
           }
         }
-      }
-      unsigned big = __ballot_sync(0xffffffffu, v < n && e - s > SMALL_DEG);
-      while (big) {
-        int bl = __ffs(big) - 1;
-        big &= big - 1;
-        int vb = __shfl_sync(0xffffffffu, v, bl);
-        int sb = __shfl_sync(0xffffffffu, s, bl), eb = __shfl_sync(0xffffffffu, e, bl);
-        bool done = false;
-        for (int c0 = sb; c0 < eb && !done; c0 += 32) {
-          int j = c0 + lane;
-          int u = -1;
-          u64 rs = 0;
-          if (j < eb) { u = ld_ro(p.cadj + j); rs = vld(p.rowst + u); S(SS_GYEDGES)++; }
-          unsigned cand = __ballot_sync(0xffffffffu, u >= 0 && mu_of(rs) == -1);
-          while (cand && !done) {
-            int l = __ffs(cand) - 1;
-            cand &= cand - 1;
-            int ok = 0;
-            if (lane == l) {
-              ok = atomicCAS(p.rowst + u, rs, pack(vb, psi_of(rs))) == rs;
-              if (ok) vst(p.colst + vb, pack(u, 0));
+        unsigned big = __ballot_sync(0xffffffffu, v[k] >= 0 && e[k] - s[k] > SMALL_DEG && !done[k] && pos[k] < e[k]);
+        while (big) {  // the rest of a long list: the whole warp
+          int bl = __ffs(big) - 1;
+          big &= big - 1;
+          int vb = __shfl_sync(0xffffffffu, v[k], bl);
+          int sb = __shfl_sync(0xffffffffu, pos[k], bl), eb = __shfl_sync(0xffffffffu, e[k], bl);
+          bool dn = false;
+          for (int c0 = sb; c0 < eb && !dn; c0 += 32) {
+            int j = c0 + lane;
+            int uu = -1;
+            u64 rr = 0;
+            if (j < eb) { uu = ld_ro(p.cadj + j); rr = vld(p.rowst + uu); S(SS_GYEDGES)++; }
+            unsigned cand = __ballot_sync(0xffffffffu, uu >= 0 && mu_of(rr) == -1);
+            while (cand && !dn) {
+              int l = __ffs(cand) - 1;
+              cand &= cand - 1;
+              int ok = 0;
+              if (lane == l) {
+                ok = atomicCAS(p.rowst + uu, rr, pack(vb, psi_of(rr))) == rr;
+                if (ok) vst(p.colst + vb, pack(uu, 0));
+              }
+              dn = __shfl_sync(0xffffffffu, ok, l);
             }
-            done = __shfl_sync(0xffffffffu, ok, l);
           }
         }
       }
@@ -450,15 +568,44 @@ struct Solver {
   // solve mode: rows without any edge can never be matched nor reach a column, so
   // they stay out of U (their count goes to ring counter j+1)
   __device__ void build_unmatched_rows(int *U, int j) {
+    // RB rows per thread per tile, all loads of a stage issued before any is used
+    // (the vertex-state loads are volatile asm: written one item at a time they
+    // would run as RB dependent round trips); one reservation per tile
+    constexpr int RB = 8;
     long long iso = 0;
-    for (int t = blockIdx.x * NT; t < m; t += gridDim.x * NT) {
-      int u = t + threadIdx.x;
-      bool f = u < m && mu_of(vld(p.rowst + u)) == -1;
-      if (f && p.mode == MODE_SOLVE && ld_ro(p.rptr + u) == ld_ro(p.rptr + u + 1)) { f = false; iso++; }
-      int tot, r = cta_rank<NT>(f, sm.w, &tot);
+    for (long long t = (long long)blockIdx.x * NT * RB; t < m; t += (long long)gridDim.x * NT * RB) {
+      int u[RB];
+      u64 w[RB];
+      int rs[RB], re[RB];
+#pragma unroll
+      for (int k = 0; k < RB; k++) {
+        const long long x = t + k * NT + threadIdx.x;
+        u[k] = x < m ? (int)x : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < RB; k++) w[k] = u[k] >= 0 ? vld(p.rowst + u[k]) : 0ull;
+      const bool need_deg = p.mode == MODE_SOLVE;
+#pragma unroll
+      for (int k = 0; k < RB; k++) {
+        const bool f = u[k] >= 0 && mu_of(w[k]) == -1 && need_deg;
+        rs[k] = f ? ld_ro(p.rptr + u[k]) : 0;
+        re[k] = f ? ld_ro(p.rptr + u[k] + 1) : 1;
+      }
+      int cnt = 0;
+      unsigned fm = 0;
+#pragma unroll
+      for (int k = 0; k < RB; k++) {
+        bool f = u[k] >= 0 && mu_of(w[k]) == -1;
+        if (f && need_deg && rs[k] == re[k]) { f = false; iso++; }
+        if (f) { fm |= 1u << k; cnt++; }
+      }
+      int tot, r = cta_scan<NT>(cnt, sm.w, &tot);
       if (threadIdx.x == 0) sm.qbase = tot ? (int)atomicAdd(ring_now(j), (u32)tot) : 0;
       __syncthreads();
-      if (f) U[sm.qbase + r] = u;
+      r += sm.qbase;
+#pragma unroll
+      for (int k = 0; k < RB; k++)
+        if (fm >> k & 1) U[r++] = u[k];
     }
     add_count(iso, j + 1);
   }
@@ -497,7 +644,7 @@ struct Solver {
     if (GRID && lvl > 0 && MCM_FINE) tmark(101, curlen);
     for (int t = cta<GRID>() * per_tile; t < curlen; t += ncta<GRID>() * per_tile) {
       int i = t + (int)threadIdx.x / G;
-      int u = -1, s = 0, e = 0;
+      int u = -1, s = 0, e = 0, cont = 0;
       if (lvl == 0) {
         u = (i < curlen) ? ld_cg(cur0 + i) : -1;
         bool keep = false;
@@ -516,10 +663,10 @@ struct Solver {
         if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
       } else if (i < curlen) {
         int4 q = ld_q(cur4 + i);
-        u = q.x; s = q.y; e = q.z;
+        u = q.x; s = q.y; e = q.z; cont = q.w;
       }
       if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(102, 0);
-      if (u >= 0 && gl == 0) { S(SS_GRROWS)++; S(SS_GREDGES) += e - s; }
+      if (u >= 0 && gl == 0) { S(SS_GRROWS) += !cont; S(SS_GREDGES) += e - s; }
       const bool big = u >= 0 && G < 32 && e - s > BIG_DEG;
       if (u >= 0 && !big) expand(s + gl, e, G, lc, lr, next, ncnt, guard, gcnt, G >= 4);
       unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
@@ -586,11 +733,11 @@ struct Solver {
         int w = mu_of(cs[k]);
         if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: mu(v) > -1 and mu(mu(v)) = v
           vst(p.rowst + w, pack(v[k], lr));
-          stage(make_int4(w, rs[k], re[k], 0), next, ncnt);
+          stage_row(w, rs[k], re[k], next, ncnt);
         } else {
           S(SS_FREE)++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
-          if (mu_of(cs[k]) != -2) atomicAdd(ring_now(2), 1u);  // an alive unmatched column got its label
+          if (mu_of(cs[k]) != -2) count_free();  // an alive unmatched column got its label
         }
       }
     }
@@ -660,11 +807,11 @@ struct Solver {
         if (w >= 0) { rw = vld(p.rowst + w); rs = ld_ro(p.rptr + w); re = ld_ro(p.rptr + w + 1); }
         if (w >= 0 && mu_of(rw) == v) {  // matched: its mate joins the next level
           vst(p.rowst + w, pack(v, lr));
-          stage(make_int4(w, rs, re, 0), next, ncnt);
+          stage_row(w, rs, re, next, ncnt);
         } else {
           S(SS_FREE)++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v;
-          if (w != -2) atomicAdd(ring_now(2), 1u);
+          if (w != -2) count_free();
         }
       }
       flush(next, ncnt);
@@ -761,24 +908,56 @@ struct Solver {
   // race (Ap(i) = v still unmatched => Ac(i) <- v, l.3-6), then mark the slot's
   // column active in this loop (l.8-11, reading R5: after the if/else).
   __device__ __forceinline__ int fix_slot(int i, int *Ac, const int *Ap, int loop) {
-    int v = ld_wl(Ap + i);
     int a;
-    if (v != -1 && col_unmatched(v)) {
-      Ac[i] = v;
-      a = v;
-    } else {
-      a = ld_wl(Ac + i);
-    }
-    if (a != -1) vst(p.iA + a, loop);
+    fix_slots<1>(i, i + 1, Ac, Ap, loop, &a);
     return a;
+  }
+  // slots i0 .. i0+RB-1 (< hi); val[k] = the slot's column after the fix, or -1.
+  // Loads are issued stage by stage for all RB slots (Ap and Ac, then the rolled-
+  // back columns' words, then their mates' words).
+  template <int RB>
+  __device__ __forceinline__ void fix_slots(int i0, int hi, int *Ac, const int *Ap, int loop, int *val) {
+    int v[RB], a[RB];
+    u64 cw[RB], rw[RB];
+#pragma unroll
+    for (int k = 0; k < RB; k++) {
+      const bool ok = i0 + k < hi;
+      v[k] = ok ? ld_wl(Ap + i0 + k) : -1;
+      a[k] = ok ? ld_wl(Ac + i0 + k) : -1;
+    }
+#pragma unroll
+    for (int k = 0; k < RB; k++) cw[k] = v[k] != -1 ? vld(p.colst + v[k]) : 0ull;
+#pragma unroll
+    for (int k = 0; k < RB; k++) rw[k] = (v[k] != -1 && mu_of(cw[k]) >= 0) ? vld(p.rowst + mu_of(cw[k])) : 0ull;
+#pragma unroll
+    for (int k = 0; k < RB; k++) {
+      if (v[k] != -1) {  // l.3-6: roll back a push that lost its race (R1: v still unmatched)
+        const int c = mu_of(cw[k]);
+        if (c == -1 || (c >= 0 && mu_of(rw[k]) != v[k])) {
+          Ac[i0 + k] = v[k];
+          a[k] = v[k];
+        }
+      }
+      if (a[k] != -1) vst(p.iA + a[k], loop);  // l.8-11 (R5)
+      val[k] = a[k];
+    }
   }
 
   template <bool GRID>
   __device__ void fix_plain(int len, int *Ac, const int *Ap, int loop, int j) {
     long long cnt = 0;
-    for (int t = cta<GRID>() * NT; t < len; t += ncta<GRID>() * NT) {
-      int i = t + threadIdx.x;
-      if (i < len) cnt += fix_slot(i, Ac, Ap, loop) != -1;
+    if (GRID && len > 2 * NT * ncta<GRID>()) {  // wide: 4 slots per thread in flight
+      for (int t = cta<GRID>() * NT * 4; t < len; t += ncta<GRID>() * NT * 4) {
+        int val[4];
+        fix_slots<4>(t + (int)threadIdx.x * 4, len, Ac, Ap, loop, val);
+#pragma unroll
+        for (int k = 0; k < 4; k++) cnt += val[k] != -1;
+      }
+    } else {
+      for (int t = cta<GRID>() * NT; t < len; t += ncta<GRID>() * NT) {
+        int i = t + threadIdx.x;
+        if (i < len) cnt += fix_slot(i, Ac, Ap, loop) != -1;
+      }
     }
     S(SS_SLOTS) += cnt;
     add_count(cnt, j);
@@ -790,12 +969,14 @@ struct Solver {
   // than HUGE_DEG to the whole CTA (a straggler column would otherwise hold up the
   // phase: C2's dense "rail" columns have 2,000 rows).  Every scan takes a
   // (label, position) minimum per step with the early exit at psi(v)-1 (R11).
+  // iaw: iA(wb) when the caller loaded it already (push_wide), else IA_LOAD
+  static constexpr int IA_LOAD = -0x7fffffff - 1;
   __device__ __forceinline__ void push_finalize(int i, int v, u64 cs, u64 best, int ub, int wb, int loop, u32 base,
-                                                int *Ac, int *Ap) {
+                                                int *Ac, int *Ap, int iaw = IA_LOAD) {
     // (dead columns are counted for the early-stop GR target, R22)
     int psimin = best == ~0ull ? INF : (int)(best >> 32);
     if (psimin < INF) {                                 // l.12
-      if (wb == -1 || vld(p.iA + wb) != loop) {      // l.13
+      if (wb == -1 || (iaw == IA_LOAD ? vld(p.iA + wb) : iaw) != loop) {  // l.13
         vst(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
         vst(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
         Ap[i] = wb;                                     // l.18 (R3)
@@ -809,7 +990,8 @@ struct Solver {
       Ac[i] = -1;                                       // l.21
       Ap[i] = -1;                                       // l.22
       S(SS_DEAD)++;
-      atomicAdd(&p.ctrl->ndead, 1u);
+      cg::coalesced_group g = cg::coalesced_threads();  // published once per tile (push)
+      if (g.thread_rank() == 0) atomicAdd(&sm.nd, (u32)g.size());
     }
   }
 
@@ -817,6 +999,10 @@ struct Solver {
   __device__ void push(int len, int *Ac, int *Ap, int loop, u32 base) {
     const int lane = lane_id();
     const int G = pick_group(len, ncta<GRID>() * NT);
+    if (GRID && len > 2 * NT * ncta<GRID>()) {
+      push_wide<GRID>(len, Ac, Ap, loop, base);
+      return;
+    }
     const int gl = lane & (G - 1), per_tile = NT / G;
     const unsigned gmask = group_mask(G);
     for (int t = cta<GRID>() * per_tile; t < len; t += ncta<GRID>() * per_tile) {
@@ -861,26 +1047,151 @@ struct Solver {
         else if (i < len) Ap[i] = -1;                   // l.24
       }
       __syncthreads();
+      // deferred long lists: with more than HUGE_CTA of them, those of at most
+      // HUGE_WARP entries get a warp each (in parallel), the rest the whole CTA each
+      // (a warp walks ~128 entries per round trip, the CTA ~2048: R-MAT hub columns
+      // of 10^5 entries on one warp held the phase for ~1.2 ms)
       const int nh = min(sm.nhuge, MAXHUGE);
-      if (nh <= HUGE_CTA) {
-        for (int h = 0; h < nh; h++) {  // a few very long lists: the whole CTA each
+      if (nh > HUGE_CTA) {
+        for (int h = warp_id(); h < nh; h += NWARP) {
           const int4 hq = sm.huge[h];
-          u64 hb;
-          int hu, hw;
-          scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
-          if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
-        }
-      } else {
-        for (int h = warp_id(); h < nh; h += NWARP) {  // many: one warp each, in parallel
-          const int4 hq = sm.huge[h];
+          if (hq.w - hq.z > HUGE_WARP) continue;
           u64 hb;
           int hu, hw;
           scan(hq.z, hq.w, lane, 32, 0xffffffffu, sm.huget[h], base, hb, hu, hw);
           if (lane == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
         }
       }
+      for (int h = 0; h < nh; h++) {
+        const int4 hq = sm.huge[h];
+        if (nh > HUGE_CTA && hq.w - hq.z <= HUGE_WARP) continue;
+        u64 hb;
+        int hu, hw;
+        scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
+        if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+      }
       __syncthreads();
-      if (threadIdx.x == 0) sm.nhuge = 0;
+      if (threadIdx.x == 0) {
+        sm.nhuge = 0;
+        if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
+      }
+      __syncthreads();
+    }
+  }
+  // PUSHKRNL on a wide worklist (more than two slots per thread): PB slots per
+  // thread per tile, each stage's loads issued for all of them before any is used
+  // -- Ac, then the column words and bounds, then the first KB neighbours and their
+  // row words, then iA of the displaced columns -- so a thread keeps PB chains in
+  // flight.  Short lists (<= BIG_DEG) whose first KB neighbours do not reach
+  // psi(v)-1 continue alone (scan from s+KB, positions kept relative to s, so the
+  // first-minimum tie-break of R11 is unchanged); longer lists take the warp / CTA
+  // paths of push().
+  template <bool GRID>
+  __device__ void push_wide(int len, int *Ac, int *Ap, int loop, u32 base) {
+    constexpr int PB = 4;
+    const int lane = lane_id();
+    for (int t = cta<GRID>() * NT * PB; t < len; t += ncta<GRID>() * NT * PB) {
+      int i[PB], v[PB], s[PB], e[PB], tg[PB];
+      u64 cs[PB];
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        i[k] = t + k * NT + (int)threadIdx.x;
+        v[k] = i[k] < len ? ld_wl(Ac + i[k]) : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : 0ull;
+        s[k] = v[k] >= 0 ? ld_ro(p.cptr + v[k]) : 0;
+        e[k] = v[k] >= 0 ? ld_ro(p.cptr + v[k] + 1) : 0;
+      }
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        const int psiv = labf(psi_of(cs[k]), base, fl_c);
+        if (p.dead_skip && psiv >= INF) e[k] = s[k];  // R19
+        tg[k] = psiv - 1;
+      }
+      int x[PB][KB];
+      u64 rs[PB][KB];
+#pragma unroll
+      for (int k = 0; k < PB; k++)
+#pragma unroll
+        for (int q = 0; q < KB; q++)
+          x[k][q] = (v[k] >= 0 && e[k] - s[k] <= BIG_DEG && s[k] + q < e[k]) ? ld_ro(p.cadj + s[k] + q) : -1;
+#pragma unroll
+      for (int k = 0; k < PB; k++)
+#pragma unroll
+        for (int q = 0; q < KB; q++) rs[k][q] = x[k][q] >= 0 ? vld(p.rowst + x[k][q]) : 0ull;
+      u64 best[PB];
+      int ub[PB], wb[PB];
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        best[k] = ~0ull;
+        ub[k] = -1;
+        wb[k] = -1;
+#pragma unroll
+        for (int q = 0; q < KB; q++) {
+          if (x[k][q] < 0) continue;
+          S(SS_SCAN)++;
+          const int l = labf(psi_of(rs[k][q]), base, fl_r);
+          const u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)q) : ~0ull;
+          if (kk < best[k]) { best[k] = kk; ub[k] = x[k][q]; wb[k] = mu_of(rs[k][q]); }
+        }
+      }
+#pragma unroll
+      for (int k = 0; k < PB; k++) {  // short lists longer than KB without a hit: the rest, alone
+        const int sk = s[k], ek = e[k];
+        if (v[k] >= 0 && ek - sk > KB && ek - sk <= BIG_DEG && !(best[k] != ~0ull && (int)(best[k] >> 32) == tg[k])) {
+          u64 b2;
+          int u2, w2;
+          scan(sk + KB, ek, 0, 1, 1u << lane, tg[k], base, b2, u2, w2);
+          if (b2 != ~0ull) b2 += KB;  // position relative to s
+          if (b2 < best[k]) { best[k] = b2; ub[k] = u2; wb[k] = w2; }
+        }
+      }
+      // longer lists: the whole warp (BIG_DEG < deg <= HUGE_DEG) or the CTA (deferred)
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        bool huge = v[k] >= 0 && e[k] - s[k] > HUGE_DEG;
+        if (huge) {
+          int q = atomicAdd(&sm.nhuge, 1);
+          if (q < MAXHUGE) { sm.huge[q] = make_int4(i[k], v[k], s[k], e[k]); sm.hugec[q] = cs[k]; sm.huget[q] = tg[k]; }
+          else huge = false;
+        }
+        if (huge) v[k] = -2;  // finalized by the CTA pass
+        unsigned bigm = __ballot_sync(0xffffffffu, v[k] >= 0 && e[k] - s[k] > BIG_DEG);
+        while (bigm) {
+          const int bl = __ffs(bigm) - 1;
+          bigm &= bigm - 1;
+          const int sb = __shfl_sync(0xffffffffu, s[k], bl), eb = __shfl_sync(0xffffffffu, e[k], bl);
+          const int tb = __shfl_sync(0xffffffffu, tg[k], bl);
+          u64 b2;
+          int u2, w2;
+          scan(sb, eb, lane, 32, 0xffffffffu, tb, base, b2, u2, w2);
+          if (lane == bl) { best[k] = b2; ub[k] = u2; wb[k] = w2; }
+        }
+      }
+      int ia[PB];
+#pragma unroll
+      for (int k = 0; k < PB; k++) ia[k] = (v[k] >= 0 && best[k] != ~0ull && wb[k] != -1) ? vld(p.iA + wb[k]) : -1;
+#pragma unroll
+      for (int k = 0; k < PB; k++) {
+        if (v[k] >= 0) push_finalize(i[k], v[k], cs[k], best[k], ub[k], wb[k], loop, base, Ac, Ap, ia[k]);
+        else if (v[k] == -1 && i[k] < len) Ap[i[k]] = -1;  // l.24
+      }
+      __syncthreads();
+      const int nh = min(sm.nhuge, MAXHUGE);
+      for (int h = 0; h < nh; h++) {
+        const int4 hq = sm.huge[h];
+        u64 hb;
+        int hu, hw;
+        scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
+        if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+      }
+      __syncthreads();
+      if (threadIdx.x == 0) {
+        sm.nhuge = 0;
+        if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
+      }
       __syncthreads();
     }
   }
@@ -1256,7 +1567,11 @@ struct Solver {
     trace(3, c.len);
     if (!GRID || (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) || p.compact_every || c.compact_next) {
       if (lead()) S(SS_SLOTS) += c.len;
-      int r1 = compact_pass1<GRID>(c.len, [&](int i) { return fix_slot(i, Ac, Ap, lp); }, Tb(c), Ac);
+      int r1 = (GRID && c.len > 2 * NT * ncta<GRID>())
+                   ? compact_pass1<GRID, 4>(c.len, [&](int i0, int hi, int *val) { fix_slots<4>(i0, hi, Ac, Ap, lp, val); },
+                                            Tb(c), Ac)
+                   : compact_pass1<GRID, 1>(c.len, [&](int i0, int hi, int *val) { fix_slots<1>(i0, hi, Ac, Ap, lp, val); },
+                                            Tb(c), Ac);
         barrier<GRID, false>();
       if (ncta<GRID>() > 1) {
         c.len = compact_pass2<GRID>(c.len, Tb(c), Ac, r1);
@@ -1436,6 +1751,7 @@ struct Solver {
     Ctrl *x = p.ctrl;
     if (threadIdx.x == 0 && blockIdx.x == 0) {
       serial_fix_push(c, reason);
+      if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
       x->ho_reason = reason;
       x->ho_ph = ph;
       const long long *src = reinterpret_cast<const long long *>(&c);
@@ -1533,7 +1849,7 @@ struct Solver {
     int *Ac = p.wl0, *Ap = p.wl1;
     int *U = p.qa, *T = p.qb;
     int4 *Qa = Q4(0), *Qb = Q4(1);
-    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
+    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; sm.nd = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
     for (int k = 0; k < SS_N; k++) sm.ts[k][threadIdx.x] = 0;
     if (threadIdx.x < 2) sm.lvc[threadIdx.x] = 0;
     init_state();
@@ -1545,7 +1861,15 @@ struct Solver {
     debug_check(1, -1, nullptr, 0);
     // unmatched rows -> U; unmatched columns (increasing id) -> Ac (R12)
     build_unmatched_rows(U, 0);
-    int run1 = compact_pass1<true>(n, [&](int v) { return col_unmatched(v) ? v : -1; }, T, Ac);
+    // isolated columns stay out of the worklist and count as dead (R25), except in
+    // serial mode (the simulator's worklist holds every unmatched column, R12) and
+    // in G-PR-First (no worklist: its loop tests and kills them itself)
+    const bool skip_iso = p.mode == MODE_SOLVE && !((F & F_SERIAL) && p.serial) && !((F & F_FIRST) && p.variant == 1);
+    long long iso_c = 0;
+    int run1 = compact_pass1<true, 8>(
+        n, [&](int i0, int hi, int *val) { iso_c += cols_unmatched<8>(i0, hi, val, skip_iso); }, T, Ac);
+    iso_c = cta_sum<NT>(iso_c, sm.red);
+    if (threadIdx.x == 0 && iso_c) atomicAdd(&p.ctrl->ndead, (u32)iso_c);
     barrier<true>();
     int ulen = (int)ring_prev(0);
     n_iso = (int)ring_prev(1);  // isolated rows (never in U)
