@@ -171,6 +171,21 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
  * cardinality (>= 0) or a negative error code.  Synchronises `stream` once. */
 int64_t mcm_solve(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t *cmatch);
 
+/* One call from HOST memory to HOST memory (the end-to-end path): copies the CSR
+ * indptr (m+1) / indices (nnz) from the HOST straight into the workspace's CSR
+ * copy, validates and transposes it there (as mcm_create), solves (as mcm_solve)
+ * and copies the matching into the HOST arrays rmatch (m) / cmatch (n).  All
+ * copies are enqueued on `stream` (asynchronous when the host arrays are pinned)
+ * and the call synchronises `stream` twice (validation result, final
+ * cardinality).  workspace: DEVICE, >= mcm_workspace_bytes(m, n, nnz, o); no
+ * handle outlives the call.  o: NULL = defaults; init = MCM_INIT_GIVEN is not
+ * supported here (MCM_EINVAL).  stats (may be NULL) receives the solve's
+ * statistics.  Returns the cardinality or a negative error code (the CSR checks
+ * of mcm_create apply). */
+int64_t mcm_match_host(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz,
+                       void *workspace, size_t ws_bytes, mcm_stream_t stream, const mcm_options_t *o,
+                       int32_t *rmatch, int32_t *cmatch, mcm_stats_t *stats);
+
 /* Global relabel (Alg. 4/5) of a given matching: rmatch (m) and cmatch
  * (n) are DEVICE inputs with the paper's mu conventions (column entries may be
  * stale or -2; rows are authoritative); writes psi_row (m) and psi_col

@@ -13,13 +13,15 @@ Names follow include/mcm.h:
 * :class:`Matcher` -- ``mcm_create`` / ``mcm_solve`` / ``mcm_global_relabel`` /
   ``mcm_set_options`` / ``mcm_get_stats`` / ``mcm_destroy`` on one graph
 * :func:`solve` -- create + solve in one call: ``(card, rmatch, cmatch)``
+* :func:`match_host` -- ``mcm_match_host``: host CSR in, host matching out (the
+  end-to-end path: H2D, create, solve and D2H in one C call)
 """
 from __future__ import annotations
 
 import ctypes
 import os
 
-__all__ = ["Options", "Stats", "Matcher", "solve", "lib", "mcm_default_options", "mcm_workspace_bytes",
+__all__ = ["Options", "Stats", "Matcher", "solve", "match_host", "lib", "mcm_default_options", "mcm_workspace_bytes",
            "MCMError", "LIB_PATH"]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -97,6 +99,8 @@ def lib():
         L.mcm_create.restype = ctypes.c_int
         L.mcm_solve.argtypes = [vp, vp, vp, vp]
         L.mcm_solve.restype = i64
+        L.mcm_match_host.argtypes = [vp, vp, i32, i32, i64, vp, sz, vp, P(Options), vp, vp, P(Stats)]
+        L.mcm_match_host.restype = i64
         L.mcm_global_relabel.argtypes = [vp, vp, vp, vp, vp, vp, P(i64)]
         L.mcm_global_relabel.restype = i64
         L.mcm_gap_relabel.argtypes = [vp, vp, vp, vp]
@@ -262,3 +266,45 @@ def solve(indptr, indices, m: int, n: int, stream=None, **opts):
         return mt.solve(stream=stream)
     finally:
         mt.close()
+
+
+def _host_i32(t, name, length):
+    torch = _torch()
+    if not isinstance(t, torch.Tensor) or t.is_cuda:
+        raise TypeError(f"{name} must be a CPU (preferably pinned) tensor")
+    if t.dtype != torch.int32 or not t.is_contiguous() or t.numel() != length:
+        raise ValueError(f"{name}: need a contiguous int32 tensor of {length} elements")
+    return ctypes.c_void_p(t.data_ptr() if length else 0)
+
+
+def match_host(indptr, indices, m: int, n: int, workspace=None, rmatch=None, cmatch=None, stream=None, device=None,
+               **opts):
+    """``mcm_match_host``: CSR in HOST memory (int32 CPU tensors, pinned for
+    asynchronous copies) -> ``(card, rmatch, cmatch, stats)`` with the matching in
+    HOST int32 tensors.  The device work (validation, transpose, solve) runs in
+    libmcm.so on ``device`` (default: the current CUDA device); ``workspace`` (a
+    CUDA uint8 tensor of at least mcm_workspace_bytes) is allocated when None."""
+    torch = _torch()
+    m, n, nnz = int(m), int(n), int(indices.numel())
+    o = mcm_default_options(**opts)
+    need = mcm_workspace_bytes(m, n, nnz, o)
+    if need == 0:
+        raise MCMError(MCM_EINVAL, "mcm_workspace_bytes")
+    dev = torch.device("cuda", torch.cuda.current_device()) if device is None else torch.device(device)
+    if workspace is None:
+        workspace = torch.empty(need, dtype=torch.uint8, device=dev)
+    if not workspace.is_cuda or workspace.numel() < need:
+        raise ValueError(f"workspace: need a CUDA uint8 tensor of at least {need} bytes")
+    if rmatch is None:
+        rmatch = torch.empty(m, dtype=torch.int32, pin_memory=True)
+    if cmatch is None:
+        cmatch = torch.empty(n, dtype=torch.int32, pin_memory=True)
+    st = Stats()
+    with torch.cuda.device(workspace.device):
+        card = lib().mcm_match_host(_host_i32(indptr, "indptr", m + 1), _host_i32(indices, "indices", nnz), m, n, nnz,
+                                    ctypes.c_void_p(workspace.data_ptr()), workspace.numel(), _stream_ptr(stream),
+                                    ctypes.byref(o), _host_i32(rmatch, "rmatch", m), _host_i32(cmatch, "cmatch", n),
+                                    ctypes.byref(st))
+    if card < 0:
+        raise MCMError(int(card), "mcm_match_host")
+    return int(card), rmatch, cmatch, st.as_dict()

@@ -24,7 +24,7 @@ constexpr int MAX_CTAS = 4096;
 size_t align256(size_t x) { return (x + 255) & ~(size_t)255; }
 
 struct Layout {
-  size_t ctrl, ovf, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, dbg, total;
+  size_t ctrl, ovf, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, outr, outc, dbg, total;
   int hist_len;
 };
 
@@ -52,6 +52,8 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   L.bsum = take(sizeof(int) * ((size_t)n / SCAN_B + 2));
   L.hist_len = (int)std::min<long long>((long long)m + n + 2, 1 << 20);
   L.hist = take(sizeof(int) * (size_t)L.hist_len);
+  L.outr = take(sizeof(int) * (size_t)m);  // mcm_match_host: device copy of the matching
+  L.outc = take(sizeof(int) * (size_t)n);
   L.dbg = take(sizeof(int) * ((size_t)n + 1) + (getenv("MCM_TRACE") ? (size_t)atoi(getenv("MCM_TRACE")) * 24 : 0));
   L.total = o;
   return L;
@@ -258,8 +260,11 @@ static int check_opts(const mcm_options_t *o) {
   return MCM_OK;
 }
 
-int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz, void *workspace,
-               size_t ws_bytes, mcm_stream_t stream_, const mcm_options_t *o, mcm_handle_t *out) {
+// from_host: indptr / indices are HOST arrays, copied straight into the workspace's
+// CSR copy (mcm_match_host); else DEVICE arrays (mcm_create)
+static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz,
+                       void *workspace, size_t ws_bytes, mcm_stream_t stream_, const mcm_options_t *o,
+                       mcm_handle_t *out, bool from_host) {
   mcm_ctx *h = nullptr;
   if (!out || !sizes_ok(m, n, nnz) || !indptr || (nnz > 0 && !indices) || !workspace) return MCM_EINVAL;
   if (check_opts(o) != MCM_OK) return MCM_EINVAL;
@@ -286,20 +291,27 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   char *ws = h->ws;
   Ctrl *ctrl = (Ctrl *)(ws + L.ctrl);
   int *err = &ctrl->err;
+  int *rptr = (int *)(ws + L.rptr), *radj = (int *)(ws + L.radj);
   CK(cudaMemsetAsync(ctrl, 0, sizeof(Ctrl), st));
+  if (from_host) {  // H2D straight into the CSR copy, validated there
+    CK(cudaMemcpyAsync(rptr, indptr, sizeof(int) * ((size_t)m + 1), cudaMemcpyHostToDevice, st));
+    if (nnz) CK(cudaMemcpyAsync(radj, indices, sizeof(int) * (size_t)nnz, cudaMemcpyHostToDevice, st));
+  }
+  const int32_t *vp = from_host ? rptr : indptr, *vi = from_host ? radj : indices;
   int vb = (int)std::min<long long>(std::max<long long>((nnz + 255) / 256, (m + 255) / 256 + 1), 4096);
-  k_validate<<<vb, 256, 0, st>>>(indptr, indices, m, n, nnz, err);
+  k_validate<<<vb, 256, 0, st>>>(vp, vi, m, n, nnz, err);
   CK(cudaGetLastError());
   int herr = 0;
   CK(cudaMemcpyAsync(&herr, err, sizeof(int), cudaMemcpyDeviceToHost, st));
   CK(cudaStreamSynchronize(st));
   if (herr) return MCM_EINVAL;
 
-  int *rptr = (int *)(ws + L.rptr), *radj = (int *)(ws + L.radj);
   int *cptr = (int *)(ws + L.cptr), *cadj = (int *)(ws + L.cadj);
   int *cnt = (int *)(ws + L.q[0]), *cursor = (int *)(ws + L.q[1]), *bsum = (int *)(ws + L.bsum);
-  CK(cudaMemcpyAsync(rptr, indptr, sizeof(int) * ((size_t)m + 1), cudaMemcpyDeviceToDevice, st));
-  if (nnz) CK(cudaMemcpyAsync(radj, indices, sizeof(int) * (size_t)nnz, cudaMemcpyDeviceToDevice, st));
+  if (!from_host) {
+    CK(cudaMemcpyAsync(rptr, indptr, sizeof(int) * ((size_t)m + 1), cudaMemcpyDeviceToDevice, st));
+    if (nnz) CK(cudaMemcpyAsync(radj, indices, sizeof(int) * (size_t)nnz, cudaMemcpyDeviceToDevice, st));
+  }
   // CSC by counting sort (Gamma(v) for the push, Alg. 9 l.6)
   CK(cudaMemsetAsync(cnt, 0, sizeof(int) * ((size_t)n + 1), st));
   if (nnz) {
@@ -333,8 +345,15 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   return MCM_OK;
 }
 
+int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz, void *workspace,
+               size_t ws_bytes, mcm_stream_t stream, const mcm_options_t *o, mcm_handle_t *out) {
+  return create_impl(indptr, indices, m, n, nnz, workspace, ws_bytes, stream, o, out, false);
+}
+
+// host_r / host_c (optional): HOST buffers the outputs are copied into before the
+// single synchronisation
 static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin, const int32_t *cin, int32_t *out_r,
-                      int32_t *out_c) {
+                      int32_t *out_c, int32_t *host_r = nullptr, int32_t *host_c = nullptr) {
   if (h->poisoned) return MCM_ECUDA;
   int dev = -1;
   CK(cudaGetDevice(&dev));
@@ -426,6 +445,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = sizeof(Smem); cfg.stream = st;
   cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
   CK(cudaLaunchKernelEx(&cfg, kern, p));
+  if (host_r && h->m) CK(cudaMemcpyAsync(host_r, out_r, sizeof(int32_t) * (size_t)h->m, cudaMemcpyDeviceToHost, st));
+  if (host_c && h->n) CK(cudaMemcpyAsync(host_c, out_c, sizeof(int32_t) * (size_t)h->n, cudaMemcpyDeviceToHost, st));
   CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));
   CK(cudaStreamSynchronize(st));
   const Ctrl &c = h->host_ctrl;
@@ -459,6 +480,21 @@ int64_t mcm_solve(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t 
   if (!h) return MCM_EINVAL;
   if ((h->m > 0 && !rmatch) || (h->n > 0 && !cmatch)) return MCM_EINVAL;
   return launch(h, (cudaStream_t)stream, MODE_SOLVE, rmatch, cmatch, rmatch, cmatch);
+}
+
+int64_t mcm_match_host(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t n, int64_t nnz,
+                       void *workspace, size_t ws_bytes, mcm_stream_t stream, const mcm_options_t *o, int32_t *rmatch,
+                       int32_t *cmatch, mcm_stats_t *stats) {
+  if ((m > 0 && !rmatch) || (n > 0 && !cmatch)) return MCM_EINVAL;
+  if (o && o->init == MCM_INIT_GIVEN) return MCM_EINVAL;  // no device copy of a given matching on this path
+  mcm_handle_t h = nullptr;
+  int rc = create_impl(indptr, indices, m, n, nnz, workspace, ws_bytes, stream, o, &h, true);
+  if (rc != MCM_OK) return rc;
+  std::unique_ptr<mcm_ctx> guard(h);
+  int32_t *dr = (int32_t *)(h->ws + h->L.outr), *dc = (int32_t *)(h->ws + h->L.outc);
+  int64_t card = launch(h, (cudaStream_t)stream, MODE_SOLVE, dr, dc, dr, dc, rmatch, cmatch);
+  if (stats) *stats = h->stats;
+  return card;
 }
 
 int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,

@@ -21,7 +21,7 @@ def test_header_declares_the_boundary():
     names = declared_functions()
     for f in ["mcm_create", "mcm_solve", "mcm_set_k", "mcm_get_stats", "mcm_destroy", "mcm_strerror", "mcm_abi_sizes",
               "mcm_gap_relabel",
-              "mcm_default_options", "mcm_workspace_bytes", "mcm_global_relabel", "mcm_set_options"]:
+              "mcm_default_options", "mcm_workspace_bytes", "mcm_global_relabel", "mcm_set_options", "mcm_match_host"]:
         assert f in names
 
 
@@ -49,6 +49,7 @@ def test_host_only_calls():
     assert b"workspace" in L.mcm_strerror(-3)
     # NULL handle / NULL args -> MCM_EINVAL without touching CUDA
     assert L.mcm_solve(None, None, None, None) == -1
+    assert L.mcm_match_host(None, None, 4, 4, 0, None, 0, None, None, None, None, None) == -1
     assert L.mcm_destroy(None) == -1
     assert L.mcm_set_k(None, 0.5) == -1
     h = ctypes.c_void_p()

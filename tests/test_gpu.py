@@ -188,6 +188,27 @@ def test_rejects_malformed_csr():
         pkg.Matcher(ip, torch.tensor([0, 1], dtype=torch.int32, device=DEV), 2, 2)
 
 
+def test_match_host_end_to_end():
+    """mcm_match_host: host CSR in, host matching out (the bench's e2e path)."""
+    for g in (synth.config("C1", 0.5), synth.config("C2", 0.01), synth.hall_violator(3000, 150, 41, 9),
+              synth.from_pairs(4, 6, [], []), synth.from_pairs(0, 0, [], [])):
+        ip = torch.from_numpy(np.ascontiguousarray(g.indptr)).pin_memory()
+        ix = torch.from_numpy(np.ascontiguousarray(g.indices)).pin_memory()
+        card, rm, cm, st = pkg.match_host(ip, ix, g.m, g.n)
+        mm = g.mm if g.mm is not None else oracle.hopcroft_karp(g)[0]
+        assert card == mm and st["card"] == card, (g.name, card, mm)
+        assert not rm.is_cuda and not cm.is_cuda
+        assert oracle.check_matching(g, rm.numpy(), cm.numpy()) == card
+        assert oracle.konig_cover(g, rm.numpy(), cm.numpy())[0] == card
+    # pageable host memory works too; malformed CSR is rejected before any solve
+    g = synth.config("C1", 0.2)
+    card, rm, cm, _ = pkg.match_host(torch.from_numpy(g.indptr.copy()), torch.from_numpy(g.indices.copy()), g.m, g.n,
+                                     rmatch=torch.empty(g.m, dtype=torch.int32), cmatch=torch.empty(g.n, dtype=torch.int32))
+    assert card == oracle.hopcroft_karp(g)[0]
+    with pytest.raises(pkg.MCMError):
+        pkg.match_host(torch.tensor([0, 1, 2], dtype=torch.int32), torch.tensor([0, 7], dtype=torch.int32), 2, 2)
+
+
 def test_race_stress():
     """Every column races for the same rows (K_{a,b}, empty M0), repeated."""
     for g in (synth.complete(128, 128), synth.complete(300, 40), synth.complete(40, 300), synth.grid_double_cover(30)):
