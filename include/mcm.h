@@ -118,6 +118,11 @@ typedef struct {
   int32_t variant;      /* 0 (default): G-PR (Alg. 7, active-column worklist);
                            1: G-PR-First (Alg. 3 + Alg. 6: every column
                            tested every loop; the Fig. 1 ablation) */
+  int32_t tail_chain;   /* single-CTA tail with at most 16 active columns: each column's warp
+                           runs a chain of double pushes (the displaced column is pushed next
+                           by the same warp, its row claimed by CAS) instead of one push per
+                           loop -- a build addition (R26); 0 = the paper's one push
+                           per column per loop; default 256 = maximum pushes per chain */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 

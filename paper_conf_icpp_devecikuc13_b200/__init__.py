@@ -55,6 +55,7 @@ class Options(ctypes.Structure):
         ("bu_div", ctypes.c_int32),
         ("scan_rot", ctypes.c_int32),
         ("variant", ctypes.c_int32),
+        ("tail_chain", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]
 

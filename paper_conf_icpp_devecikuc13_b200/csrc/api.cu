@@ -237,6 +237,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->compact_every = 0;
   o->grid_ctas = 0;
   o->max_loops = 0;
+  o->tail_chain = 256;
 }
 
 static bool sizes_ok(int32_t m, int32_t n, int64_t nnz) {
@@ -269,7 +270,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
     return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
-  if (o->variant < 0 || o->variant > 1 || o->bu_div < 0) return MCM_EINVAL;
+  if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -400,6 +401,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.gr_early = o.gr_early;
   p.serial = o.serial;
   p.variant = o.variant;
+  p.tail_chain = o.tail_chain;
   p.bu_div = o.bu_div;
   p.scan_rot = o.serial ? 0 : o.scan_rot;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either

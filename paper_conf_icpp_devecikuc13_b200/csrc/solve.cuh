@@ -84,6 +84,7 @@ struct Params {
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
+  int tail_chain;          // single-CTA tail, <= NWARP active columns: max pushes per chain (0: off)
   int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
   int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
   long long max_loops;
@@ -120,6 +121,7 @@ struct Smem {
   int huget[MAXHUGE];
   int nhuge;
   u32 nd;                  // push: columns declared dead in this tile (-> Ctrl::ndead)
+  int chmax;               // push_chain: longest chain of the phase
   int qcnt, qbase, tmp;
 };
 
@@ -1195,6 +1197,74 @@ struct Solver {
       __syncthreads();
     }
   }
+  // Push chains (single-CTA tail, at most NWARP active columns; reading R26, a
+  // build addition).  In the paper's loop a double push hands the displaced column
+  // w to the next loop, so an augmenting path of length L costs ~L/2 loops, each a
+  // fix phase + a push phase (~4.4 us in the tail): C2's last augmentations walk
+  // paths of 400-900 BFS levels that way.  Here one warp per slot performs the same
+  // push operations (Alg. 9 l.4-18: first minimum-label neighbour, labels psimin+1 /
+  // psimin+2) back to back: after displacing w it pushes w itself.  The row is
+  // claimed with a CAS on its {mu, psi} word (re-read at gpu scope, so the
+  // comparison is against L2's value), which makes every displacement exclusive --
+  // the role the iA test and the rollback play for the atomic-free loop -- so the
+  // slot leaves Ac(i) = -1 and Ap(i) = its current column (or -1 when the path
+  // reached an unmatched row or the column died): the next fix step then marks
+  // exactly the unfinished chains active and rolls nothing back.
+  // Returns the longest chain (pushes), CTA-uniform: the caller advances `loop` by
+  // it, so the GR schedule (iterGR = loop + k * maxLevel, counted in push rounds)
+  // sees the same number of push rounds as the one-push-per-loop schedule -- without
+  // that, a chain circling on stale labels ran ~5 * 10^4 pushes between two GRs.
+  __device__ int push_chain(int len, int *Ac, int *Ap, u32 base) {
+    const int i = warp_id(), lane = lane_id();
+    if (i < len) {
+      int cur = ld_wl(Ac + i), left = -1, retry = 0, step = 0;
+      while (cur >= 0) {
+        if (step >= p.tail_chain || retry > 8) { left = cur; break; }
+        const u64 cs = vld(p.colst + cur);
+        const int psiv = labf(psi_of(cs), base, fl_c);
+        const int s = ld_ro(p.cptr + cur);
+        int e = ld_ro(p.cptr + cur + 1);
+        if (p.dead_skip && psiv >= INF) e = s;  // R19
+        u64 best;
+        int ub, wb;
+        scan(s, e, lane, 32, 0xffffffffu, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
+        const int psimin = best == ~0ull ? INF : (int)(best >> 32);
+        if (psimin >= INF) {  // l.19-22: dead
+          if (lane == 0) {
+            vst(p.colst + cur, pack(-2, psi_of(cs)));
+            S(SS_DEAD)++;
+            atomicAdd(&sm.nd, 1u);
+          }
+          break;
+        }
+        int ok = 0;
+        if (lane == 0) {
+          const u64 now = ld_rlx(p.rowst + ub);  // gpu scope: L2's current word
+          if (mu_of(now) == wb && labf(psi_of(now), base, fl_r) == psimin)
+            ok = atomicCAS(p.rowst + ub, now, pack(cur, base + (u32)psimin + 2u)) == now;  // l.14, l.17
+          if (ok) {
+            vst(p.colst + cur, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
+            S(SS_PUSH)++;
+          }
+        }
+        if (!__shfl_sync(0xffffffffu, ok, 0)) { retry++; continue; }  // the row changed: scan again
+        retry = 0;
+        step++;
+        cur = wb;  // -1: single push, the path is complete
+      }
+      if (lane == 0) {
+        Ac[i] = -1;
+        Ap[i] = left;
+        atomicMax(&sm.chmax, step);
+      }
+    }
+    __syncthreads();
+    const int mx = sm.chmax;
+    if (threadIdx.x == 0 && sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
+    __syncthreads();
+    if (threadIdx.x == 0) sm.chmax = 0;
+    return mx;
+  }
   // scan() with the whole CTA: KB*NT neighbours per step; CTA-wide (label, position)
   // minimum through shared memory; returns the result in every thread.
   __device__ void scan_cta(int s, int e, int target, u32 base, u64 &best, int &bu, int &bw) {
@@ -1251,8 +1321,9 @@ struct Solver {
   // rot: the scan starts at position s + rot and wraps around (option scan_rot, a
   // free tie-break in parallel mode, R11: contenders for one low-label row spread
   // over the equally low rows instead of blocking each other)
+  // fresh: row words at gpu scope (L2), for a push chain re-scanning after a lost CAS
   __device__ __forceinline__ void scan(int s, int e, int gl, int G, unsigned gmask, int target, u32 base, u64 &best,
-                                       int &bu, int &bw, int rot = 0) {
+                                       int &bu, int &bw, int rot = 0, bool fresh = false) {
     best = ~0ull;
     bu = -1;
     bw = -1;
@@ -1268,7 +1339,7 @@ struct Solver {
         x[k] = jj < e ? ld_ro(p.cadj + s + q) : -1;
       }
 #pragma unroll
-      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
+      for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? (fresh ? ld_rlx(p.rowst + x[k]) : vld(p.rowst + x[k])) : 0ull;
       u64 key = ~0ull;
       int kx = -1, kw = -1;
 #pragma unroll
@@ -1599,11 +1670,18 @@ struct Solver {
     trace(4, c.len);
     fl_r = c.floor_r;
     fl_c = c.floor_c;
-    push<GRID>(c.len, Ac, Ap, lp, cur);
+    long long adv = 1;  // push rounds of this loop (R26: a chain counts its pushes)
+    if (!GRID && p.tail_chain > 0 && p.tail_ctas == 1 && c.len <= NWARP) {
+      adv = max(1, push_chain(c.len, Ac, Ap, cur));
+      if (c.iterGR > c.loop && adv > c.iterGR - c.loop) adv = c.iterGR - c.loop;  // land on iterGR / gapAt
+      if (c.gapAt > c.loop && adv > c.gapAt - c.loop) adv = c.gapAt - c.loop;
+    } else {
+      push<GRID>(c.len, Ac, Ap, lp, cur);
+    }
     barrier<GRID, false>();
     if (GRID) debug_check(4, c.loop, nullptr, 0);
-    c.ac0 ^= 1;  // l.18: swap Ac and Ap
-    c.loop++;    // l.19
+    c.ac0 ^= 1;      // l.18: swap Ac and Ap
+    c.loop += adv;   // l.19
     if (lead()) { if (GRID) L().loops++; else L().tail_loops++; }
     if (lead()) L().ns_loop += (long long)(tnow() - l0);
     return true;
@@ -1849,7 +1927,7 @@ struct Solver {
     int *Ac = p.wl0, *Ap = p.wl1;
     int *U = p.qa, *T = p.qb;
     int4 *Qa = Q4(0), *Qb = Q4(1);
-    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; sm.nd = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
+    if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; sm.nd = 0; sm.chmax = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
     for (int k = 0; k < SS_N; k++) sm.ts[k][threadIdx.x] = 0;
     if (threadIdx.x < 2) sm.lvc[threadIdx.x] = 0;
     init_state();
