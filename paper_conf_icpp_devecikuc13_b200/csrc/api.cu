@@ -402,6 +402,9 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.serial = o.serial;
   p.variant = o.variant;
   p.tail_chain = o.tail_chain;
+  // worklists of at most this many slots run as push chains (lanes per slot from the
+  // count); MCM_CHAIN_SLOTS: analysis knob
+  p.chain_slots = getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 16;
   p.bu_div = o.bu_div;
   p.scan_rot = o.serial ? 0 : o.scan_rot;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either

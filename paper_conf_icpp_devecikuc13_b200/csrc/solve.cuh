@@ -35,7 +35,8 @@ constexpr int MAXHUGE = 32;      // CTA-wide push list per tile
 constexpr int HUGE_CTA = 4;      // at most this many per tile: one CTA-wide scan each; more: a warp each ...
 constexpr int HUGE_WARP = 8192;  // ... unless longer than this
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
-constexpr int SPLIT = 1024;      // GR: a frontier row's adjacency is split into ranges of at most this many
+constexpr int SPLIT = 1024;
+constexpr int CHAIN_SLOTS = 128; // tail push chains (R26) for worklists of at most this many slots      // GR: a frontier row's adjacency is split into ranges of at most this many
 
 enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
 
@@ -84,7 +85,8 @@ struct Params {
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
-  int tail_chain;          // single-CTA tail, <= NWARP active columns: max pushes per chain (0: off)
+  int tail_chain;          // single-CTA tail, <= chain_slots active columns: max pushes per chain (0: off)
+  int chain_slots;
   int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
   int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
   long long max_loops;
@@ -1197,7 +1199,7 @@ struct Solver {
       __syncthreads();
     }
   }
-  // Push chains (single-CTA tail, at most NWARP active columns; reading R26, a
+  // Push chains (single-CTA tail, at most chain_slots active columns; reading R26, a
   // build addition).  In the paper's loop a double push hands the displaced column
   // w to the next loop, so an augmenting path of length L costs ~L/2 loops, each a
   // fix phase + a push phase (~4.4 us in the tail): C2's last augmentations walk
@@ -1215,7 +1217,10 @@ struct Solver {
   // sees the same number of push rounds as the one-push-per-loop schedule -- without
   // that, a chain circling on stale labels ran ~5 * 10^4 pushes between two GRs.
   __device__ int push_chain(int len, int *Ac, int *Ap, u32 base) {
-    const int i = warp_id(), lane = lane_id();
+    const int lane = lane_id();
+    const int G = pick_group(len, NT), gl = lane & (G - 1), lead_lane = lane & ~(G - 1);
+    const unsigned gmask = group_mask(G);
+    const int i = (int)threadIdx.x / G;
     if (i < len) {
       int cur = ld_wl(Ac + i), left = -1, retry = 0, step = 0;
       while (cur >= 0) {
@@ -1227,10 +1232,10 @@ struct Solver {
         if (p.dead_skip && psiv >= INF) e = s;  // R19
         u64 best;
         int ub, wb;
-        scan(s, e, lane, 32, 0xffffffffu, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
+        scan(s, e, gl, G, gmask, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
         const int psimin = best == ~0ull ? INF : (int)(best >> 32);
         if (psimin >= INF) {  // l.19-22: dead
-          if (lane == 0) {
+          if (gl == 0) {
             vst(p.colst + cur, pack(-2, psi_of(cs)));
             S(SS_DEAD)++;
             atomicAdd(&sm.nd, 1u);
@@ -1238,7 +1243,7 @@ struct Solver {
           break;
         }
         int ok = 0;
-        if (lane == 0) {
+        if (gl == 0) {
           const u64 now = ld_rlx(p.rowst + ub);  // gpu scope: L2's current word
           if (mu_of(now) == wb && labf(psi_of(now), base, fl_r) == psimin)
             ok = atomicCAS(p.rowst + ub, now, pack(cur, base + (u32)psimin + 2u)) == now;  // l.14, l.17
@@ -1247,12 +1252,12 @@ struct Solver {
             S(SS_PUSH)++;
           }
         }
-        if (!__shfl_sync(0xffffffffu, ok, 0)) { retry++; continue; }  // the row changed: scan again
+        if (!__shfl_sync(gmask, ok, lead_lane)) { retry++; continue; }  // the row changed: scan again
         retry = 0;
         step++;
         cur = wb;  // -1: single push, the path is complete
       }
-      if (lane == 0) {
+      if (gl == 0) {
         Ac[i] = -1;
         Ap[i] = left;
         atomicMax(&sm.chmax, step);
@@ -1671,7 +1676,7 @@ struct Solver {
     fl_r = c.floor_r;
     fl_c = c.floor_c;
     long long adv = 1;  // push rounds of this loop (R26: a chain counts its pushes)
-    if (!GRID && p.tail_chain > 0 && p.tail_ctas == 1 && c.len <= NWARP) {
+    if (!GRID && p.tail_chain > 0 && p.tail_ctas == 1 && c.len <= p.chain_slots) {
       adv = max(1, push_chain(c.len, Ac, Ap, cur));
       if (c.iterGR > c.loop && adv > c.iterGR - c.loop) adv = c.iterGR - c.loop;  // land on iterGR / gapAt
       if (c.gapAt > c.loop && adv > c.gapAt - c.loop) adv = c.gapAt - c.loop;
