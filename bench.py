@@ -138,6 +138,30 @@ def algorithmic_bytes(st, m, n, nnz):
     return int(b)
 
 
+def sector_bytes(st, m, n, nnz):
+    """The same counters priced at the memory system's granularity: a random
+    4- or 8-byte access moves a 32-byte sector (SURVEY.md §8(d) "sector-level
+    reality"); coalesced streams move their own bytes.  A model, not a measurement
+    (DESIGN.md §6): it tells how far a solve is from the bound its access pattern
+    allows, which the algorithmic bytes above cannot.
+      push, per processed column: Ac 4 + column word 32 + bounds 32 + adjacency 32
+        + iA 32 + stores 68; per scanned neighbour: 4 + row word 32
+      fix step, per slot: Ap/Ac 8 + column word 32 + mate's row word 32 + iA 32
+      GR: per frontier entry 16 + first adjacency sector 32; per adjacency entry
+        4 + column word 32 + CAS 32; per labelled column: mate's row word 32 +
+        bounds 32 + label store 32 + staged entry 16
+      greedy: per column 16; per scanned entry 4 + row word 32 + claim 32
+      FIXMATCHING: 12 n + 8 m + 32 per matched pair
+    """
+    processed = st["pushes"] + st["blocked"] + st["dead"]
+    b = 200 * processed + 36 * st["edges_scanned"]
+    b += 104 * st["slots"]
+    b += 48 * st["gr_rows"] + 68 * st["gr_edges"] + 112 * st["gr_cols"]
+    b += 16 * n + 68 * st["greedy_edges"]
+    b += 12 * n + 8 * m + 32 * st["init_card"]
+    return int(b)
+
+
 def setup_bytes(m, n, nnz):
     """mcm_create: validate (4(m+1) + 4 nnz) + copy (2 x (4(m+1) + 4 nnz)) + count (4 nnz
     + 4 nnz atomics) + scan (3 x 4n) + scatter (4(m+1) + 4 nnz + 4 nnz atomics + 4 nnz)."""
@@ -255,6 +279,7 @@ def run_ours(args, rank, world, local_rank):
     peaks = _peaks()
     hbm_peak = peaks["hbm_gbs"] if peaks else 6650.0
     alg = algorithmic_bytes(stats, g.m, g.n, g.nnz)
+    sb_ = sector_bytes(stats, g.m, g.n, g.nnz)
     achieved = alg / (t_solve * 1e-3) / 1e9  # GB/s of the solve kernel
     traffic = None
     tp = os.path.join(ROOT, "profiles", f"ncu_traffic_{args.config}.json")
@@ -297,13 +322,16 @@ def run_ours(args, rank, world, local_rank):
             "traffic": traffic,
             "algorithmic_bytes_per_launch": alg,
             "peak_source": "MEASURED_PEAKS.json hbm_gbs" if peaks else "fallback B200_PROFILING.md",
+            "l2_sector_model": {"bytes": sb_, "achieved": sb_ / (t_solve * 1e-3) / 1e9,
+                             "frac": sb_ / (t_solve * 1e-3) / 1e9 / hbm_peak},
             "latency": {"grid_barriers": stats["grid_barriers"], "loops": stats["loops"],
                         "gr_levels": stats["gr_levels"], "us_per_grid_barrier_measured": 1.27,
                         "barrier_floor_ms": stats["grid_barriers"] * 1.27e-3},
         },
         "solve_stats": {k: stats[k] for k in ("loops", "gr_count", "gr_levels", "pushes", "blocked", "dead",
                                               "edges_scanned", "slots", "shrinks", "guard_reactivated",
-                                              "tail_loops", "grid_barriers", "ms_init", "ms_gr", "ms_loop",
+                                              "tail_loops", "grid_barriers", "gr_rows", "gr_edges", "gr_cols",
+                                              "greedy_edges", "init_card", "ms_init", "ms_gr", "ms_loop",
                                               "ms_total", "grid_ctas")},
         "clocks": clk,
         "e2e": {"value": nnz_total / (t_e2e_max * 1e-3), "unit": "edges/s",

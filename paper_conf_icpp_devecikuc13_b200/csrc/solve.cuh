@@ -643,6 +643,34 @@ struct Solver {
                            int *Uout, u32 *ucnt, int *guard, u32 *gcnt) {
     const int lane = lane_id();
     const u32 lc = base + lvl + 1, lr = base + lvl + 2;
+    if (GRID && lvl > 0 && curlen > 2 * NT * ncta<GRID>()) {
+      // wide level: two frontier entries per thread per tile, their adjacency
+      // expanded as one list in batches of 2*KB (twice the loads in flight of a
+      // one-entry tile; the kernel's register budget caps the batch)
+      for (int t = cta<GRID>() * 2 * NT; t < curlen; t += ncta<GRID>() * 2 * NT) {
+        const int i0 = t + (int)threadIdx.x, i1 = i0 + NT;
+        int4 q0 = i0 < curlen ? ld_q(cur4 + i0) : make_int4(-1, 0, 0, 0);
+        int4 q1 = i1 < curlen ? ld_q(cur4 + i1) : make_int4(-1, 0, 0, 0);
+        if (q0.x >= 0) { S(SS_GRROWS) += !q0.w; S(SS_GREDGES) += q0.z - q0.y; }
+        if (q1.x >= 0) { S(SS_GRROWS) += !q1.w; S(SS_GREDGES) += q1.z - q1.y; }
+        const bool big0 = q0.x >= 0 && q0.z - q0.y > BIG_DEG, big1 = q1.x >= 0 && q1.z - q1.y > BIG_DEG;
+        expand_pair(big0 || q0.x < 0 ? 0 : q0.z - q0.y, q0.y, big1 || q1.x < 0 ? 0 : q1.z - q1.y, q1.y, lc, lr, next,
+                    ncnt, guard, gcnt);
+#pragma unroll
+        for (int h = 0; h < 2; h++) {
+          const int4 q = h ? q1 : q0;
+          unsigned bigm = __ballot_sync(0xffffffffu, h ? big1 : big0);
+          while (bigm) {  // long lists: the whole warp
+            int bl = __ffs(bigm) - 1;
+            bigm &= bigm - 1;
+            int sb = __shfl_sync(0xffffffffu, q.y, bl), eb = __shfl_sync(0xffffffffu, q.z, bl);
+            expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt, false);
+          }
+        }
+        flush(next, ncnt);
+      }
+      return;
+    }
     const int G = pick_group(curlen, ncta<GRID>() * NT);
     const int gl = lane & (G - 1), per_tile = NT / G;
     if (GRID && lvl > 0 && MCM_FINE) tmark(101, curlen);
@@ -742,6 +770,53 @@ struct Solver {
           S(SS_FREE)++;
           if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
           if (mu_of(cs[k]) != -2) count_free();  // an alive unmatched column got its label
+        }
+      }
+    }
+  }
+  // expand() over the concatenation of two adjacency ranges radj[s0, s0+d0) and
+  // radj[s1, s1+d1), 2*KB entries per batch, wide-level claiming (only CAS winners
+  // load their mate)
+  __device__ __forceinline__ void expand_pair(int d0, int s0, int d1, int s1, u32 lc, u32 lr, int4 *next, u32 *ncnt,
+                                              int *guard, u32 *gcnt) {
+    constexpr int B = 2 * KB;
+    const int tot = d0 + d1;
+    for (int o = 0; o < tot; o += B) {
+      int v[B];
+      u64 cs[B], old[B], rw[B];
+      int rs[B], re[B];
+#pragma unroll
+      for (int k = 0; k < B; k++) {
+        const int x = o + k;
+        v[k] = x < d0 ? ld_ro(p.radj + s0 + x) : (x < tot ? ld_ro(p.radj + s1 + (x - d0)) : -1);
+      }
+#pragma unroll
+      for (int k = 0; k < B; k++) cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : ~0ull;
+#pragma unroll
+      for (int k = 0; k < B; k++) {
+        const bool try_ = v[k] >= 0 && psi_of(cs[k]) < gr_base;
+        old[k] = try_ ? atomicCAS(p.colst + v[k], cs[k], pack(mu_of(cs[k]), lc)) : ~cs[k];
+      }
+#pragma unroll
+      for (int k = 0; k < B; k++) {
+        const int w = mu_of(cs[k]);
+        const bool go = old[k] == cs[k] && w >= 0;
+        rw[k] = go ? vld(p.rowst + w) : 0ull;
+        rs[k] = go ? ld_ro(p.rptr + w) : 0;
+        re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
+      }
+#pragma unroll
+      for (int k = 0; k < B; k++) {
+        if (old[k] != cs[k]) continue;  // not claimed by this thread
+        S(SS_GRCOLS)++;
+        const int w = mu_of(cs[k]);
+        if (w >= 0 && mu_of(rw[k]) == v[k]) {  // matched: its mate joins the next level
+          vst(p.rowst + w, pack(v[k], lr));
+          stage_row(w, rs[k], re[k], next, ncnt);
+        } else {
+          S(SS_FREE)++;
+          if (guard) guard[atomicAdd(gcnt, 1u)] = v[k];
+          if (mu_of(cs[k]) != -2) count_free();
         }
       }
     }
