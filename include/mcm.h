@@ -123,6 +123,10 @@ typedef struct {
                            by the same warp, its row claimed by CAS) instead of one push per
                            loop -- a build addition (R26); 0 = the paper's one push
                            per column per loop; default 256 = maximum pushes per chain */
+  int32_t grid_chain;   /* the same push chains for grid loops with at most one active column per
+                           two threads (rows claimed by CAS at gpu scope, re-scanned at gpu scope
+                           after a lost claim); default 128 = maximum pushes per chain; 0 = the
+                           paper's one push per column per loop */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
 } mcm_options_t;
 

@@ -56,6 +56,7 @@ class Options(ctypes.Structure):
         ("scan_rot", ctypes.c_int32),
         ("variant", ctypes.c_int32),
         ("tail_chain", ctypes.c_int32),
+        ("grid_chain", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
     ]
 

@@ -238,6 +238,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->grid_ctas = 0;
   o->max_loops = 0;
   o->tail_chain = 256;
+  o->grid_chain = 128;
 }
 
 static bool sizes_ok(int32_t m, int32_t n, int64_t nnz) {
@@ -270,7 +271,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
     return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
-  if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0) return MCM_EINVAL;
+  if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0 || o->grid_chain < 0) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -405,14 +406,17 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   // worklists of at most this many slots run as push chains (lanes per slot from the
   // count); MCM_CHAIN_SLOTS: analysis knob
   p.chain_slots = getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 16;
+  p.grid_chain = o.grid_chain;
+  p.grid_chain_div = getenv("MCM_GRID_CHAIN_DIV") ? atoi(getenv("MCM_GRID_CHAIN_DIV")) : 2;
   p.bu_div = o.bu_div;
   p.scan_rot = o.serial ? 0 : o.scan_rot;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either
     p.tail_max = 0;
     p.serial = 0;
   }
-  if (o.serial) {  // the simulator's schedule: complete GRs, no tail, no adaptive compaction
+  if (o.serial) {  // the simulator's schedule: complete GRs, no tail, no adaptive compaction, no chains
     p.tail_max = 0;
+    p.grid_chain = 0;
     p.gr_early = 0;
     p.compact_adapt = 0;
     p.compact_every = 0;

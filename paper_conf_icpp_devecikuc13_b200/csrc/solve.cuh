@@ -87,6 +87,8 @@ struct Params {
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
   int tail_chain;          // single-CTA tail, <= chain_slots active columns: max pushes per chain (0: off)
   int chain_slots;
+  int grid_chain;          // grid loops of <= 1/grid_chain_div slot per thread: max pushes per chain (0: off)
+  int grid_chain_div;
   int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
   int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
   long long max_loops;
@@ -1291,15 +1293,20 @@ struct Solver {
   // it, so the GR schedule (iterGR = loop + k * maxLevel, counted in push rounds)
   // sees the same number of push rounds as the one-push-per-loop schedule -- without
   // that, a chain circling on stale labels ran ~5 * 10^4 pushes between two GRs.
-  __device__ int push_chain(int len, int *Ac, int *Ap, u32 base) {
+  // GRID: the slots spread over all CTAs (grid_chain); the longest chain goes to
+  // ring counter 5 and the caller reads it after the barrier (returns 0).
+  template <bool GRID>
+  __device__ int push_chain(int len, int *Ac, int *Ap, u32 base, int cap) {
     const int lane = lane_id();
-    const int G = pick_group(len, NT), gl = lane & (G - 1), lead_lane = lane & ~(G - 1);
+    const int G = pick_group(len, ncta<GRID>() * NT), gl = lane & (G - 1), lead_lane = lane & ~(G - 1);
     const unsigned gmask = group_mask(G);
-    const int i = (int)threadIdx.x / G;
+    const int per_tile = NT / G;
+    for (int t = cta<GRID>() * per_tile; t < len; t += ncta<GRID>() * per_tile) {
+    const int i = t + (int)threadIdx.x / G;
     if (i < len) {
       int cur = ld_wl(Ac + i), left = -1, retry = 0, step = 0;
       while (cur >= 0) {
-        if (step >= p.tail_chain || retry > 8) { left = cur; break; }
+        if (step >= cap || retry > 8) { left = cur; break; }
         const u64 cs = vld(p.colst + cur);
         const int psiv = labf(psi_of(cs), base, fl_c);
         const int s = ld_ro(p.cptr + cur);
@@ -1338,7 +1345,16 @@ struct Solver {
         atomicMax(&sm.chmax, step);
       }
     }
+    }
     __syncthreads();
+    if (GRID) {
+      if (threadIdx.x == 0) {
+        if (sm.chmax) atomicMax(ring_now(5), (u32)sm.chmax);
+        if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
+        sm.chmax = 0;
+      }
+      return 0;
+    }
     const int mx = sm.chmax;
     if (threadIdx.x == 0 && sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
     __syncthreads();
@@ -1751,14 +1767,22 @@ struct Solver {
     fl_r = c.floor_r;
     fl_c = c.floor_c;
     long long adv = 1;  // push rounds of this loop (R26: a chain counts its pushes)
+    const bool chain_grid = GRID && p.grid_chain > 0 && (long long)c.len * p.grid_chain_div <= (long long)ncta<GRID>() * NT;
     if (!GRID && p.tail_chain > 0 && p.tail_ctas == 1 && c.len <= p.chain_slots) {
-      adv = max(1, push_chain(c.len, Ac, Ap, cur));
-      if (c.iterGR > c.loop && adv > c.iterGR - c.loop) adv = c.iterGR - c.loop;  // land on iterGR / gapAt
-      if (c.gapAt > c.loop && adv > c.gapAt - c.loop) adv = c.gapAt - c.loop;
+      adv = max(1, push_chain<false>(c.len, Ac, Ap, cur, p.tail_chain));
+    } else if (chain_grid) {
+      push_chain<true>(c.len, Ac, Ap, cur, p.grid_chain);
     } else {
       push<GRID>(c.len, Ac, Ap, lp, cur);
     }
-    barrier<GRID, false>();
+    if (chain_grid) {
+      barrier<GRID, true>();
+      adv = max(1, (int)ring_prev(5));
+    } else {
+      barrier<GRID, false>();
+    }
+    if (c.iterGR > c.loop && adv > c.iterGR - c.loop) adv = c.iterGR - c.loop;  // land on iterGR / gapAt
+    if (c.gapAt > c.loop && adv > c.gapAt - c.loop) adv = c.gapAt - c.loop;
     if (GRID) debug_check(4, c.loop, nullptr, 0);
     c.ac0 ^= 1;      // l.18: swap Ac and Ap
     c.loop += adv;   // l.19

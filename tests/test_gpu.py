@@ -113,7 +113,9 @@ OPTION_SETS = [
     dict(tail_max=4096, tail_f=100000), dict(tail_max=32, tail_f=32), dict(gr_early=1), dict(gr_early=1, tail_max=0),
     dict(gr_early=1, k=3.0), dict(gr_early=0), dict(variant=1), dict(variant=1, gr_early=0, k=0.3), dict(bu_div=0),
     dict(bu_div=1), dict(bu_div=100000), dict(scan_rot=1), dict(tail_chain=0), dict(tail_chain=1),
-    dict(tail_chain=1 << 30), dict(tail_chain=4, tail_max=16), dict(tail_chain=64, k=3.0),
+    dict(tail_chain=1 << 30), dict(tail_chain=4, tail_max=16), dict(tail_chain=64, k=3.0), dict(grid_chain=0),
+    dict(grid_chain=1), dict(grid_chain=1 << 30), dict(grid_chain=4, tail_max=0), dict(grid_chain=0, tail_chain=0),
+    dict(grid_chain=1000, tail_max=0, k=0.1),
 ]
 
 

@@ -27,7 +27,7 @@ STRATS = [("adaptive 0.3", dict(k=0.3)), ("adaptive 0.7", dict(k=0.7)), ("adapti
 def main():
     mode = sys.argv[1]
     cfgs = sys.argv[2:] or ["C1", "C2", "C3", "C5"]
-    base = dict(gr_early=0, compact_adapt=0) if mode == "paper" else {}
+    base = dict(gr_early=0, compact_adapt=0, tail_chain=0, grid_chain=0) if mode == "paper" else {}
     reps = int(os.environ.get("REPS", "3"))
     graphs = []
     for c in cfgs:
