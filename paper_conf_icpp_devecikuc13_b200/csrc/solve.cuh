@@ -1312,6 +1312,7 @@ struct Solver {
         const int s = ld_ro(p.cptr + cur);
         int e = ld_ro(p.cptr + cur + 1);
         if (p.dead_skip && psiv >= INF) e = s;  // R19
+        if (step > 0 && e - s > HUGE_DEG * G / 32) { left = cur; break; }  // a long list ends the chain
         u64 best;
         int ub, wb;
         scan(s, e, gl, G, gmask, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
@@ -1771,7 +1772,9 @@ struct Solver {
     if (!GRID && p.tail_chain > 0 && p.tail_ctas == 1 && c.len <= p.chain_slots) {
       adv = max(1, push_chain<false>(c.len, Ac, Ap, cur, p.tail_chain));
     } else if (chain_grid) {
-      push_chain<true>(c.len, Ac, Ap, cur, p.grid_chain);
+      // the longest chain holds the phase: shorter chains on longer worklists
+      const int cap = c.len <= 1024 ? p.grid_chain : max(8, (int)((long long)p.grid_chain * 1024 / c.len));
+      push_chain<true>(c.len, Ac, Ap, cur, min(cap, p.grid_chain));
     } else {
       push<GRID>(c.len, Ac, Ap, lp, cur);
     }
