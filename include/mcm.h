@@ -85,7 +85,7 @@ typedef struct {
   int32_t dead_skip;    /* 1 (default): an active column whose label is already
                            >= m+n dies without scanning Gamma(v) (R19). */
   int32_t tail_max;     /* worklists of at most this many slots run on the tail group
-                           (tail_ctas CTAs) instead of the whole grid (0 = off); default 256 */
+                           (tail_ctas CTAs) instead of the whole grid (0 = off); default 32 */
   int32_t tail_f;       /* GR levels whose frontier has at most this many rows run on the
                            tail group (handed back to the grid above it, to the tail below
                            tail_f/2); 0 = 2 * tail_max; default 128 */

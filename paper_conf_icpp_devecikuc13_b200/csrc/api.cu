@@ -228,7 +228,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->gap = 0;
   o->final_check = 1;
   o->dead_skip = 1;
-  o->tail_max = 256;
+  o->tail_max = 32;
   o->tail_f = 128;
   o->tail_ctas = 1;
   o->compact_adapt = 1;
@@ -405,7 +405,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_chain = o.tail_chain;
   // worklists of at most this many slots run as push chains (lanes per slot from the
   // count); MCM_CHAIN_SLOTS: analysis knob
-  p.chain_slots = getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 16;
+  p.chain_slots = getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 32;
   p.grid_chain = o.grid_chain;
   p.grid_chain_div = getenv("MCM_GRID_CHAIN_DIV") ? atoi(getenv("MCM_GRID_CHAIN_DIV")) : 2;
   p.bu_div = o.bu_div;
