@@ -212,6 +212,36 @@ def test_match_host_end_to_end():
         pkg.match_host(torch.tensor([0, 1, 2], dtype=torch.int32), torch.tensor([0, 7], dtype=torch.int32), 2, 2)
 
 
+def test_concurrent_solves_on_streams():
+    """Several persistent solves at once (one host thread, stream and handle each,
+    a quarter of the CTAs each): the batch mode of bench.py --config C5."""
+    import threading
+
+    graphs = [synth.config("C5", 1 / 64, index=i) for i in range(4)] + [synth.config("C2", 0.01)]
+    out = [None] * len(graphs)
+
+    def run(j):
+        g = graphs[j]
+        st = torch.cuda.Stream()
+        ip, ix = dev(g)
+        torch.cuda.synchronize()
+        mt = pkg.Matcher(ip, ix, g.m, g.n, stream=st, grid_ctas=37)
+        card, rm, cm = mt.solve(stream=st)
+        st.synchronize()
+        out[j] = (card, rm.cpu().numpy(), cm.cpu().numpy())
+        mt.close()
+
+    ths = [threading.Thread(target=run, args=(j,)) for j in range(len(graphs))]
+    for t in ths:
+        t.start()
+    for t in ths:
+        t.join()
+    for g, (card, rm, cm) in zip(graphs, out):
+        mm = g.mm if g.mm is not None else oracle.hopcroft_karp(g)[0]
+        assert card == mm, (g.name, card, mm)
+        assert oracle.check_matching(g, rm, cm) == card
+
+
 def test_race_stress():
     """Every column races for the same rows (K_{a,b}, empty M0), repeated."""
     for g in (synth.complete(128, 128), synth.complete(300, 40), synth.complete(40, 300), synth.grid_double_cover(30)):
