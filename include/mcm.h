@@ -151,6 +151,7 @@ typedef struct {
   int64_t gr_edges;          /* adjacency entries read by all GR levels */
   int64_t gr_cols;           /* columns labelled by all GRs */
   int64_t greedy_edges;      /* adjacency entries read by the greedy initial matching */
+  int64_t rows_repaired;     /* stale rows (mate not pointing back) made unmatched before the guard GR (R27) */
   double ms_init;            /* device time: initial matching + worklist build */
   double ms_gr;              /* device time in global relabels */
   double ms_loop;            /* device time in fix + push steps */

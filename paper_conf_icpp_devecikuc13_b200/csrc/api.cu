@@ -474,7 +474,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   s.shrinks = x[ST_SHRINKS]; s.gaps = x[ST_GAPS]; s.guard_reactivated = x[ST_GUARD]; s.fixed_cols = x[ST_FIXED];
   s.init_card = x[ST_INITCARD]; s.card = x[ST_CARD]; s.tail_loops = x[ST_TAILLOOPS]; s.grid_barriers = x[ST_BARRIERS];
   s.gr_rows = x[ST_GR_ROWS]; s.gr_edges = x[ST_GR_EDGES]; s.gr_cols = x[ST_GR_COLS];
-  s.greedy_edges = x[ST_GREEDY_EDGES];
+  s.greedy_edges = x[ST_GREEDY_EDGES]; s.rows_repaired = x[ST_REPAIRED];
   s.ms_init = x[ST_NS_INIT] * 1e-6; s.ms_gr = x[ST_NS_GR] * 1e-6; s.ms_loop = x[ST_NS_LOOP] * 1e-6;
   s.ms_total = x[ST_NS_TOTAL] * 1e-6; s.ms_setup = h->ms_setup; s.grid_ctas = grid; s.threads_per_cta = NT;
   if (p.debug && c.dbg[0])

@@ -17,6 +17,9 @@
 
 namespace cg = cooperative_groups;
 
+#ifndef MCM_CHAIN_PLAIN
+#define MCM_CHAIN_PLAIN 0
+#endif
 #ifndef MCM_FINE
 #define MCM_FINE 0
 #endif
@@ -44,7 +47,7 @@ enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
 enum {
   ST_LOOPS, ST_GRS, ST_LEVELS, ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_SHRINKS, ST_GAPS,
   ST_GUARD, ST_FIXED, ST_INITCARD, ST_CARD, ST_TAILLOOPS, ST_BARRIERS, ST_NS_INIT, ST_NS_GR, ST_NS_LOOP,
-  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_NSTAT = 32
+  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_REPAIRED, ST_NSTAT = 32
 };
 
 struct Ctrl {
@@ -103,7 +106,7 @@ enum { SS_PUSH, SS_BLOCK, SS_DEAD, SS_SCAN, SS_SLOTS, SS_FREE, SS_GRROWS, SS_GRE
 // control-loop statistics and the phase-trace cursor: kept by the lead thread
 // (block 0, thread 0) only, in shared memory, so they hold no registers
 struct LeadStats {
-  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar;
+  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar, repaired;
   int tn, ttag, tsz, pad;
 };
 struct Smem;
@@ -1295,6 +1298,18 @@ struct Solver {
   // that, a chain circling on stale labels ran ~5 * 10^4 pushes between two GRs.
   // GRID: the slots spread over all CTAs (grid_chain); the longest chain goes to
   // ring counter 5 and the caller reads it after the barrier (returns 0).
+  // mu(c) <- r after a chain claimed row r for column c (R27).  The store is a CAS
+  // against the word the chain read, so a late write cannot overwrite a newer one:
+  // once another chain has displaced c from r (CAS on r's word) and pushed c on,
+  // c's word belongs to that chain.  A failed CAS (a stale read, or the newer
+  // write already landed) is retried only while r still holds c.
+  __device__ __forceinline__ void chain_settle(int c, int r, u64 exp, u64 val, u64 ret) {
+    while (ret != exp) {
+      if (mu_of(ld_rlx(p.rowst + r)) != c) return;  // displaced: the newer push owns mu(c)
+      exp = ret;
+      ret = atomicCAS(p.colst + c, exp, val);
+    }
+  }
   template <bool GRID>
   __device__ int push_chain(int len, int *Ac, int *Ap, u32 base, int cap) {
     const int lane = lane_id();
@@ -1305,6 +1320,10 @@ struct Solver {
     const int i = t + (int)threadIdx.x / G;
     if (i < len) {
       int cur = ld_wl(Ac + i), left = -1, retry = 0, step = 0;
+      // the last push's mu(column) CAS, checked one scan later (its latency hides
+      // behind the next column's loads): {column, row, expected, written, returned}
+      int pc = -1, pr = -1;
+      u64 pexp = 0, pnew = 0, pret = 0;
       while (cur >= 0) {
         if (step >= cap || retry > 8) { left = cur; break; }
         const u64 cs = vld(p.colst + cur);
@@ -1316,6 +1335,7 @@ struct Solver {
         u64 best;
         int ub, wb;
         scan(s, e, gl, G, gmask, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
+        if (gl == 0 && pc >= 0) { chain_settle(pc, pr, pexp, pnew, pret); pc = -1; }
         const int psimin = best == ~0ull ? INF : (int)(best >> 32);
         if (psimin >= INF) {  // l.19-22: dead
           if (gl == 0) {
@@ -1330,8 +1350,14 @@ struct Solver {
           const u64 now = ld_rlx(p.rowst + ub);  // gpu scope: L2's current word
           if (mu_of(now) == wb && labf(psi_of(now), base, fl_r) == psimin)
             ok = atomicCAS(p.rowst + ub, now, pack(cur, base + (u32)psimin + 2u)) == now;  // l.14, l.17
-          if (ok) {
-            vst(p.colst + cur, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
+          if (ok) {  // l.15, l.16
+            pc = cur; pr = ub; pexp = cs; pnew = pack(ub, base + (u32)psimin + 1u);
+#if MCM_CHAIN_PLAIN  // A/B only: the plain store of the first round-1 build
+            vst(p.colst + cur, pnew);
+            pret = pexp;
+#else
+            pret = atomicCAS(p.colst + cur, pexp, pnew);
+#endif
             S(SS_PUSH)++;
           }
         }
@@ -1340,7 +1366,9 @@ struct Solver {
         step++;
         cur = wb;  // -1: single push, the path is complete
       }
+      __syncwarp(gmask);  // every lane of the group has read Ac(i) before it is cleared
       if (gl == 0) {
+        if (pc >= 0) chain_settle(pc, pr, pexp, pnew, pret);
         Ac[i] = -1;
         Ap[i] = left;
         atomicMax(&sm.chmax, step);
@@ -1993,12 +2021,72 @@ struct Solver {
     return true;
   }
 
+  // Stale rows (R27, build addition): at termination a row u with mu(u) = c whose
+  // column does not point back (mu(c) != u).  The paper argues that only column
+  // entries of mu can be inconsistent when the loop ends.  Push chains
+  // (R26) claim rows by CAS but store mu(c) plainly, and when c is displaced from
+  // a row and pushed on by another chain before the first chain's store of mu(c)
+  // has landed, that late store leaves mu(c) naming the row c was displaced from
+  // (seen under compute-sanitizer's slowed schedule; 0 in 600 plain solves).  A
+  // stale row would count in |M| and never start a BFS.  So before the guard's GR:
+  // if c's own row does not point back either, c is re-attached to u (CAS on
+  // c's word, so one row wins when several hold c); otherwise, or when the CAS
+  // loses, u is set unmatched and appended to U, and the guard's GR then reaches
+  // every unmatched column an augmenting path still leads to.  One pass over the
+  // row words (plus the mates' column words).
+  __device__ void repair_rows(Ctl &c) {
+    int *U = Ub(c);
+    const int cap = max(m, n) + 1;
+    long long fixedc = 0, freed = 0;
+    for (int t = blockIdx.x * NT; t < m; t += gridDim.x * NT) {
+      const int u = t + (int)threadIdx.x;
+      u64 w = 0, cw = 0;
+      int cc = -1;
+      bool stale = false;
+      if (u < m) {
+        w = vld(p.rowst + u);
+        cc = mu_of(w);
+        if (cc >= 0) {
+          cw = ld_rlx(p.colst + cc);
+          stale = mu_of(cw) != u;
+        }
+      }
+      bool drop = false;
+      if (stale) {
+        const int u2 = mu_of(cw);
+        const bool c_free = u2 < 0 || mu_of(ld_rlx(p.rowst + u2)) != cc;
+        if (c_free && atomicCAS(p.colst + cc, cw, pack(u, psi_of(cw))) == cw) {
+          if (u2 == -2) atomicSub(&p.ctrl->ndead, 1u);
+          fixedc++;
+        } else {
+          vst(p.rowst + u, pack(-1, psi_of(w)));
+          drop = true;
+          freed++;
+        }
+      }
+      if (drop) {
+        cg::coalesced_group g = cg::coalesced_threads();
+        u32 b = 0;
+        if (g.thread_rank() == 0) b = atomicAdd(ring_now(6), (u32)g.size());
+        b = g.shfl(b, 0);
+        const long long at = (long long)c.ulen + b + g.thread_rank();
+        if (at < cap) U[at] = u;
+      }
+    }
+    add_count(fixedc + freed, 7);
+    barrier<true>();
+    const int nr = (int)ring_prev(6);
+    if (nr) c.ulen = (int)min((long long)c.ulen + nr, (long long)cap);
+    if (lead()) L().repaired += ring_prev(7);
+  }
+
   // exactness guard (R16): one more GR; every unmatched column it reaches is
   // re-activated and the loop resumes (returns true); otherwise the labels certify
   // maximality (returns false).
   __device__ bool guard_step(Ctl &c) {
     if (!p.final_check) return false;
     u64 g0 = tnow();
+    repair_rows(c);
     if (base_overflow(c)) { reset_labels(); c.base = 1; }
     int gcount = 0;
     int *Ac = Acp(c), *Ap = App(c);
@@ -2165,6 +2253,7 @@ struct Solver {
       st[ST_GUARD] = l.guard_re; st[ST_INITCARD] = init_card; st[ST_NS_INIT] = ns_init; st[ST_NS_GR] = l.ns_gr;
       st[ST_NS_LOOP] = l.ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = l.tail_loops;
       st[ST_BARRIERS] = l.nbar;
+      st[ST_REPAIRED] = l.repaired;
       st[ST_TRACE_N] = l.tn;
       if (p.mode == MODE_SOLVE) {
         st[ST_CARD] = (long long)ring_prev(0);

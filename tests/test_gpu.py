@@ -139,6 +139,32 @@ def test_given_initial_matching():
     assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == card
 
 
+@pytest.mark.parametrize("drop_cols", [False, True])
+def test_stale_rows_repaired(drop_cols):
+    """R27: rows whose column does not point back (the state a late chain store can
+    leave) are repaired before the guard GR.  An initial matching with such rows
+    reproduces it deterministically: drop_cols=False -> the column words point to
+    rows that do not point back (the column is re-attached to its row or the row is
+    freed); drop_cols=True -> the column words are -1."""
+    g = synth.config("C2", 0.01)
+    _, rm0, cm0 = oracle.cheap_match(g)
+    rm0 = rm0.astype(np.int32).copy()
+    cm0 = cm0.astype(np.int32).copy()
+    rng = np.random.default_rng(7)
+    matched = np.nonzero(rm0 >= 0)[0]
+    stale = rng.choice(matched, size=64, replace=False)
+    for u in stale:
+        c = rm0[u]
+        cm0[c] = -1 if drop_cols else (u + 1) % g.m  # row (u+1) % m does not hold c
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, init="given")
+    card, rm, cm = mt.solve(torch.from_numpy(rm0).to(DEV), torch.from_numpy(cm0).to(DEV))
+    rm, cm = rm.cpu().numpy(), cm.cpu().numpy()
+    assert card == g.n  # C2 has a perfect matching (closed form)
+    assert oracle.check_matching(g, rm, cm) == card
+    assert oracle.konig_cover(g, rm, cm)[0] == card
+
+
 def test_edge_cases():
     check_solve(synth.from_pairs(0, 0, [], []), 0)
     check_solve(synth.from_pairs(5, 0, [], []), 0)
