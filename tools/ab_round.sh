@@ -1,5 +1,10 @@
-# A/B: chain mu(c) CAS (R27a) against the plain store (GPU box)
+# A/B: early-stop GR target fraction (MCM_GR_TARGET builds) on C2, C3, C5 (GPU box)
 O=gpurun_out
-for i in 1 2 3; do MCM_LIB=build_ab/plain.so python tools/variance.py C2 20 >> $O/ab_plain.txt 2>&1; python tools/variance.py C2 20 >> $O/ab_cas.txt 2>&1; done
-for c in C3 C5; do MCM_LIB=build_ab/plain.so python tools/variance.py $c 10 >> $O/ab_plain.txt 2>&1; python tools/variance.py $c 10 >> $O/ab_cas.txt 2>&1; done
-timeout 600 compute-sanitizer --tool racecheck python tools/sanitize.py quick > $O/r27b_san_racecheck.log 2>&1
+for i in 1 2 3; do for v in base t0.95 t0.8; do
+  if [ $v = base ]; then unset MCM_LIB; else export MCM_LIB=build_ab/$v.so; fi
+  python tools/ab_solve.py C2 20 $v >> $O/ab_target.txt 2>&1
+done; done
+for c in C3 C5; do for v in base t0.95 t0.8; do
+  if [ $v = base ]; then unset MCM_LIB; else export MCM_LIB=build_ab/$v.so; fi
+  python tools/ab_solve.py $c 10 $v >> $O/ab_target.txt 2>&1
+done; done

@@ -1,0 +1,26 @@
+"""Median solve time of one config with the library MCM_LIB points at (A/B of build variants, GPU box):
+    MCM_LIB=build_ab/x.so python tools/ab_solve.py C2 20 [label]"""
+import os
+import statistics
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import torch  # noqa: E402
+
+import synth  # noqa: E402
+import paper_conf_icpp_devecikuc13_b200 as pkg  # noqa: E402
+
+name, reps = sys.argv[1], int(sys.argv[2])
+label = sys.argv[3] if len(sys.argv) > 3 else os.environ.get("MCM_LIB", "in-tree")
+g = synth.config(name)
+mt = pkg.Matcher(torch.from_numpy(g.indptr).cuda(), torch.from_numpy(g.indices).cuda(), g.m, g.n)
+ts, lv, lp, gr = [], [], [], []
+for r in range(reps + 1):
+    card, _, _ = mt.solve()
+    st = mt.stats()
+    assert card == st["card"]
+    if r:
+        ts.append(st["ms_total"]); lv.append(st["gr_levels"]); lp.append(st["loops"]); gr.append(st["ms_gr"])
+print(f"{label:10s} {name} card={card} ms med={statistics.median(ts):.2f} mean={statistics.mean(ts):.2f} "
+      f"min={min(ts):.2f} max={max(ts):.2f} gr_ms med={statistics.median(gr):.2f} levels med={statistics.median(lv)} "
+      f"loops med={statistics.median(lp)}", flush=True)
