@@ -128,6 +128,12 @@ typedef struct {
                            after a lost claim); default 128 = maximum pushes per chain; 0 = the
                            paper's one push per column per loop */
   int64_t max_loops;    /* iteration cap; 0 = default (2*(m+n)+100000).  MCM_ENOCONV beyond */
+  double gr_target;     /* early-stop GR (gr_early, R22/R28): the BFS stops once this
+                           fraction of the alive unmatched columns carries a label; (0, 1];
+                           default 0.6; 1.0 = every one (R22 alone); see gr_target_min */
+  int32_t gr_target_min; /* gr_target applies only to GRs that start with at least this many
+                           alive unmatched columns (fewer: every one must be labelled);
+                           default 4096 */
 } mcm_options_t;
 
 typedef struct {

@@ -58,6 +58,8 @@ class Options(ctypes.Structure):
         ("tail_chain", ctypes.c_int32),
         ("grid_chain", ctypes.c_int32),
         ("max_loops", ctypes.c_int64),
+        ("gr_target", ctypes.c_double),
+        ("gr_target_min", ctypes.c_int32),
     ]
 
 

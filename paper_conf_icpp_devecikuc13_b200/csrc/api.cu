@@ -237,6 +237,8 @@ void mcm_default_options(mcm_options_t *o) {
   o->compact_every = 0;
   o->grid_ctas = 0;
   o->max_loops = 0;
+  o->gr_target = 0.6;
+  o->gr_target_min = 4096;
   o->tail_chain = 256;
   o->grid_chain = 128;
 }
@@ -266,6 +268,7 @@ const char *mcm_strerror(int code) {
 static int check_opts(const mcm_options_t *o) {
   if (!o) return MCM_OK;
   if (!(o->k > 0) || !std::isfinite(o->k)) return MCM_EINVAL;
+  if (!(o->gr_target > 0) || !(o->gr_target <= 1.0) || o->gr_target_min < 0) return MCM_EINVAL;
   if (o->gr_strategy != MCM_GR_ADAPTIVE && o->gr_strategy != MCM_GR_FIXED) return MCM_EINVAL;
   if (o->init < 0 || o->init > 2) return MCM_EINVAL;
   if (o->grid_ctas < 0 || o->grid_ctas > MAX_CTAS || o->tail_max < 0 || o->tail_f < 0 || o->max_loops < 0)
@@ -400,6 +403,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.compact_every = o.compact_every;
   p.compact_adapt = o.compact_adapt;
   p.gr_early = o.gr_early;
+  p.gr_target = o.gr_target;
+  p.gr_target_min = o.gr_target_min;
   p.serial = o.serial;
   p.variant = o.variant;
   p.tail_chain = o.tail_chain;

@@ -84,7 +84,8 @@ struct Params {
   int trace_cap;
   Ctrl *ctrl;
   // options
-  double k;
+  double k, gr_target;
+  int gr_target_min;
   int gr_fixed, shrink_min, init, gap, final_check, dead_skip, tail_max, compact_every, compact_adapt, gr_early;
   int serial;              // 1: fix/push by one thread in slot order (bit-exact vs the serial simulator)
   int variant;             // 0: G-PR (Alg. 7, worklist); 1: G-PR-First (Alg. 3 + Alg. 6, all columns)
@@ -1498,6 +1499,9 @@ struct Solver {
     long long card = 0, fixed = 0;
     for (int u = g; u < m; u += G) {
       int c = mu_of(vld(p.rowst + u));
+      // without the guard (final_check = 0) no repair pass ran (R27): a stale row is
+      // reported unmatched, so the output stays a valid matching
+      if (!p.final_check && c >= 0 && mu_of(vld(p.colst + c)) != u) c = -1;
       p.rmatch_out[u] = c;
       card += c >= 0;
     }
@@ -1713,6 +1717,8 @@ struct Solver {
     // carry a label.  alive unmatched = n - matched - dead; matched = m - |U|.
     c.gst.reached = (int)ring_prev(2);
     c.gst.target = early_gr() ? n - (m - n_iso - c.ulen) - (int)bcast_ld((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
+    if (p.gr_target < 1.0 && early_gr() && c.gst.target >= p.gr_target_min)  // R28
+      c.gst.target = (int)ceil(p.gr_target * (double)c.gst.target);
     if (c.gst.nlen == 0) gr_finish(c);
     else if (c.gst.reached >= c.gst.target) gr_finish(c, true);
     if (lead()) L().ns_gr += (long long)(tnow() - g0);

@@ -1,5 +1,5 @@
-"""Median solve time of one config with the library MCM_LIB points at (A/B of build variants, GPU box):
-    MCM_LIB=build_ab/x.so python tools/ab_solve.py C2 20 [label]"""
+"""Median solve time of one config (A/B of build variants via MCM_LIB, or of options; GPU box):
+    [MCM_LIB=build_ab/x.so] python tools/ab_solve.py C2 20 [label] [opt=val,...]"""
 import os
 import statistics
 import sys
@@ -12,8 +12,13 @@ import paper_conf_icpp_devecikuc13_b200 as pkg  # noqa: E402
 
 name, reps = sys.argv[1], int(sys.argv[2])
 label = sys.argv[3] if len(sys.argv) > 3 else os.environ.get("MCM_LIB", "in-tree")
+opts = {}
+if len(sys.argv) > 4:
+    for kv in sys.argv[4].split(","):
+        k, v = kv.split("=")
+        opts[k] = float(v) if "." in v else int(v)
 g = synth.config(name)
-mt = pkg.Matcher(torch.from_numpy(g.indptr).cuda(), torch.from_numpy(g.indices).cuda(), g.m, g.n)
+mt = pkg.Matcher(torch.from_numpy(g.indptr).cuda(), torch.from_numpy(g.indices).cuda(), g.m, g.n, **opts)
 ts, lv, lp, gr = [], [], [], []
 for r in range(reps + 1):
     card, _, _ = mt.solve()
