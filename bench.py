@@ -304,7 +304,7 @@ def run_ours(args, rank, world, local_rank):
         "config": {
             "workload": f"{args.config}: {CONFIG_DESC[args.config]}",
             "m": g.m, "n": g.n, "nnz": g.nnz, "mm": cards[-1], "init_card": stats["init_card"],
-            "k": args.k, "gr_strategy": "adaptive", "shrink_min": 512, "gr_target": 0.6, "gr_target_min": 4096,
+            "k": args.k, "gr_strategy": "adaptive", "shrink_min": 512, "gr_target": 0.6, "gr_target_min": 1024,
             "step": "mcm_create + mcm_solve (device-resident CSR)",
             "ms_create": t_create_max, "ms_solve": t_solve_max,
             "edges_per_s_solve_only": nnz_total / (t_solve_max * 1e-3),

@@ -133,7 +133,7 @@ typedef struct {
                            default 0.6; 1.0 = every one (R22 alone); see gr_target_min */
   int32_t gr_target_min; /* gr_target applies only to GRs that start with at least this many
                            alive unmatched columns (fewer: every one must be labelled);
-                           default 4096 */
+                           default 1024 */
 } mcm_options_t;
 
 typedef struct {

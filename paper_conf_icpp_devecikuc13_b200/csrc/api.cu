@@ -238,7 +238,7 @@ void mcm_default_options(mcm_options_t *o) {
   o->grid_ctas = 0;
   o->max_loops = 0;
   o->gr_target = 0.6;
-  o->gr_target_min = 4096;
+  o->gr_target_min = 1024;
   o->tail_chain = 256;
   o->grid_chain = 128;
 }

@@ -54,7 +54,7 @@ def test_host_only_calls():
     assert L.mcm_set_k(None, 0.5) == -1
     h = ctypes.c_void_p()
     assert L.mcm_create(None, None, 4, 4, 0, None, 0, None, None, ctypes.byref(h)) == -1
-    assert pkg.mcm_default_options().gr_target == 0.6 and pkg.mcm_default_options().gr_target_min == 4096
+    assert pkg.mcm_default_options().gr_target == 0.6 and pkg.mcm_default_options().gr_target_min == 1024
     bad = pkg.mcm_default_options(k=-1.0)
     assert L.mcm_create(None, None, 4, 4, 0, None, 0, None, ctypes.byref(bad), ctypes.byref(h)) == -1
 
