@@ -1,8 +1,8 @@
-# k x gr_target_min sweep (GPU box)
+# tail_f / bu_div sweep at the r01h defaults (GPU box)
 O=gpurun_out
-for c in C2 C4 C3 C5; do for i in 1 2; do
+for c in C2 C5 C3; do for i in 1 2; do
   r=10; [ $c = C2 ] && r=20
-  for o in k=0.4 k=0.7 k=0.7,gr_target_min=1024 k=0.4,gr_target_min=1024 k=0.7,gr_target_min=512 k=0.7,gr_target_min=1024,gr_target=0.5; do
-    timeout 300 python tools/ab_solve.py $c $r x $o 2>&1 | sed "s/^x /$o /" >> $O/r01g_sweep2.txt
+  for o in tail_f=128 tail_f=256 tail_f=512 tail_f=64 bu_div=16 bu_div=8; do
+    timeout 300 python tools/ab_solve.py $c $r x $o 2>&1 | sed "s/^x /$o /" >> $O/r01h_sweep.txt
   done
 done; done
