@@ -9,7 +9,9 @@ Contents (all cite PAPER.md, see ``oracle.c``'s header):
 
 * C (``oracle.c``): transpose, cheap matching (reading R13), GR (Alg. 2),
   sequential PR-FIFO (Alg. 1 + GR every k(m+n) pushes), Hopcroft-Karp, validity
-  checker, Konig certificate, serial G-PR simulator (Alg. 7/8/9 + Alg. 4/5).
+  checker, Konig certificate, the G-PR kernels as plain functions (INITKRNL
+  Alg. 8, SHRKRNL, PUSHKRNL Alg. 9, FIXMATCHING) and the serial G-PR simulator
+  built from them (Alg. 7/8/9 + Alg. 4/5).
 * Python: brute force by edge-subset enumeration (<= ~16 edges) and by a
   column-bitmask DP (m small); shortest alternating distances by Bellman-Ford
   over the residual digraph (an independent pin for GR).
@@ -66,6 +68,14 @@ def _get():
         lib.or_gpr_serial.restype = i64
         lib.or_gap_relabel.argtypes = [i32, i32, P32, P32, i32]
         lib.or_gap_relabel.restype = ctypes.c_int
+        lib.or_initkrnl.argtypes = [i64, i32, P32, P32, P32, P32, P32]
+        lib.or_initkrnl.restype = i64
+        lib.or_shrkrnl.argtypes = [i64, i32, P32, P32, P32, P32, P32]
+        lib.or_shrkrnl.restype = i64
+        lib.or_pushkrnl.argtypes = [i32, i32, P32, P32, i64, i32, P32, P32, P32, P32, P32, P32, P32, ctypes.c_int, P64]
+        lib.or_pushkrnl.restype = None
+        lib.or_fixmatching.argtypes = [i32, i32, P32, P32]
+        lib.or_fixmatching.restype = i64
         _lib = lib
     return _lib
 
@@ -274,3 +284,45 @@ def alternating_distances(g, mu_row, mu_col):
                 dr[w] = dc[v] + 1
                 changed = True
     return np.array(dr, np.int32), np.array(dc, np.int32)
+
+
+# ---------------------------------------------------------------- G-PR kernels as functions
+def _pad(a):
+    a = _i32(a)
+    return np.concatenate([a, [0]]).astype(np.int32)
+
+
+def initkrnl(loop, mu_row, mu_col, Ac, Ap, iA):
+    """G-PR-INITKRNL (Alg. 8) on copies -> (active_slots, Ac', iA')."""
+    Ac, iA = _pad(Ac), _pad(iA)
+    a = _get().or_initkrnl(len(Ac) - 1, int(loop), _p32(_pad(mu_row)), _p32(_pad(mu_col)), _p32(Ac), _p32(_pad(Ap)),
+                           _p32(iA))
+    return int(a), Ac[:-1], iA[:-1]
+
+
+def shrkrnl(loop, mu_row, mu_col, Ac, Ap, iA):
+    """G-PR-SHRKRNL on copies -> (len', Ac'[:len'], iA')."""
+    Ac, iA = _pad(Ac), _pad(iA)
+    ln = _get().or_shrkrnl(len(Ac) - 1, int(loop), _p32(_pad(mu_row)), _p32(_pad(mu_col)), _p32(Ac), _p32(_pad(Ap)),
+                           _p32(iA))
+    return int(ln), Ac[:ln], iA[:-1]
+
+
+def pushkrnl(g, loop, mu_row, mu_col, psi_row, psi_col, iA, Ac, dead_skip=False, csc=None):
+    """G-PR-PUSHKRNL (Alg. 9), slots in order, on copies ->
+    dict(mu_row, mu_col, psi_row, psi_col, Ac, Ap, pushes, blocked, dead)."""
+    csc = csc or transpose(g)
+    mr, mc, pr, pc, Acp = _pad(mu_row), _pad(mu_col), _pad(psi_row), _pad(psi_col), _pad(Ac)
+    Ap = np.full(len(Acp), -7, np.int32)
+    st = np.zeros(3, np.int64)
+    _get().or_pushkrnl(g.m, g.n, _p32(csc.cptr), _p32(csc.cadj), len(Acp) - 1, int(loop), _p32(mr), _p32(mc), _p32(pr),
+                       _p32(pc), _p32(_pad(iA)), _p32(Acp), _p32(Ap), int(bool(dead_skip)), _p64(st))
+    return dict(mu_row=mr[: g.m], mu_col=mc[: g.n], psi_row=pr[: g.m], psi_col=pc[: g.n], Ac=Acp[:-1], Ap=Ap[:-1],
+                pushes=int(st[0]), blocked=int(st[1]), dead=int(st[2]))
+
+
+def fixmatching(m, n, mu_row, mu_col):
+    """FIXMATCHING on a copy -> (|M|, mu_col')."""
+    mc = _pad(mu_col)
+    card = _get().or_fixmatching(int(m), int(n), _p32(_pad(mu_row)), _p32(mc))
+    return int(card), mc[:n]
