@@ -5,10 +5,18 @@
 One STEP = one pass of the whole hot path over one synthetic graph already
 resident in HBM: mcm_create (validate + copy + CSC transpose)
 followed by mcm_solve (greedy init, GRs, fix/push loop, guard, FIXMATCHING).
-Default workload: configs[1] of BASELINE.json (C2, permuted banded 1.5M x 1.5M,
-~5.47M nnz).  value = edges/s = (sum over ranks of nnz) / (max over ranks of the
-mean step time).  N > 1 (torchrun): every rank solves its own instance (seed + rank),
-no data-path collective -> "scaling": "weak".
+Default workload: C4 (R-MAT 2^23 x 2^23, 131M nnz), the largest single-GPU
+configuration of BASELINE.json (its metric names no config); C1-C3 and C5 behind
+--config.  value = edges/s = (sum over ranks of nnz) / (max over ranks of the mean
+step time).  N > 1 (torchrun): every rank solves its own instance (seed + rank), no
+data-path collective -> "scaling": "weak".
+
+Beside the step the line carries: `paper_protocol` (t_pr: the solve alone from the
+cheap matching M0 computed outside the timed region, MCM_INIT_GIVEN -- the paper
+times only the matching), `paper_config` (the paper's atomic-free loop:
+one push per column per loop, complete GRs, post-GR shrink only, k = 0.7; the
+build's push chains / early-stop GR / adaptive compaction off), `cpu_baseline`
+(the oracle's PR-FIFO and Hopcroft-Karp on the host, rank 0, N = 1).
 
 L2 (126 MB) is flushed between timed steps by writing a 512 MiB buffer outside
 the per-step CUDA events.  `e2e` repeats the measurement through the C ABI's
@@ -39,6 +47,9 @@ CONFIG_DESC = {
     "C5": "uniform 2^21 x 2^21, 16 * 2^21 samples (avg deg 16), seed 1000+i",
 }
 METRIC = "MCM solve throughput (edges/s = nnz / (create + solve time)) per graph"
+# the paper's G-PR (Alg. 7-9 with its GR schedule): no push
+# chains (R26), complete GRs (no R22 / R28 early stop), post-GR shrink only, k = 0.7
+PAPER_OPTS = dict(tail_chain=0, grid_chain=0, gr_early=0, compact_adapt=0, k=0.7)
 
 
 def _peaks():
@@ -203,6 +214,7 @@ def run_ours(args, rank, world, local_rank):
     opts = dict(k=args.k)
     need = pkg.mcm_workspace_bytes(g.m, g.n, g.nnz, pkg.mcm_default_options(**opts))
     ws = torch.empty(need, dtype=torch.uint8, device=dev)
+    launches = 0
 
     def step():
         mt = pkg.Matcher.__new__(pkg.Matcher)
@@ -237,6 +249,8 @@ def run_ours(args, rank, world, local_rank):
         e2.record(stream)
         cards.append(card)
         stats = mt.stats()
+        launches += stats["kernel_launches"]
+        used_opts = {f: getattr(mt.opts, f) for f, _ in pkg.Options._fields_}
         mt.close()
     barrier()
     wall = time.perf_counter() - t_wall
@@ -269,6 +283,10 @@ def run_ours(args, rank, world, local_rank):
         if i >= args.warmup:
             e2e_ms.append(a.elapsed_time(b))
     t_e2e = sum(e2e_ms) / len(e2e_ms)
+
+    # ---- the paper's protocol and the paper's configuration, same graph, same run
+    paper_protocol = run_paper_protocol(args, g, ip, ix, ws, rm, cm, flush, stream, opts, cards[-1])
+    paper_config = run_paper_config(args, g, ip, ix, ws, rm, cm, flush, stream, cards[-1])
 
     # ---- max over ranks (times), sum over ranks (units processed)
     t_step_max, t_e2e_max, t_solve_max, t_create_max, nnz_total = reduce_over_ranks(
@@ -304,7 +322,7 @@ def run_ours(args, rank, world, local_rank):
         "config": {
             "workload": f"{args.config}: {CONFIG_DESC[args.config]}",
             "m": g.m, "n": g.n, "nnz": g.nnz, "mm": cards[-1], "init_card": stats["init_card"],
-            "k": args.k, "gr_strategy": "adaptive", "shrink_min": 512, "gr_target": 0.6, "gr_target_min": 1024,
+            "options": used_opts,
             "step": "mcm_create + mcm_solve (device-resident CSR)",
             "ms_create": t_create_max, "ms_solve": t_solve_max,
             "edges_per_s_solve_only": nnz_total / (t_solve_max * 1e-3),
@@ -337,11 +355,93 @@ def run_ours(args, rank, world, local_rank):
         "e2e": {"value": nnz_total / (t_e2e_max * 1e-3), "unit": "edges/s",
                 "h2d_bytes_per_step": 4 * (g.m + 1 + g.nnz), "d2h_bytes_per_step": 4 * (g.m + g.n),
                 "ms_per_step": t_e2e_max},
-        "gpu_launches": args.steps * 7,
+        "gpu_launches": launches,
+        "gpu_launches_note": "kernels of the timed region, counted by libmcm at its launch sites "
+                             "(mcm_stats_t.kernel_launches: create's setup kernels + the persistent solve kernel)",
+        "paper_protocol": paper_protocol,
+        "paper_config": paper_config,
     }
+    if world > 1:
+        line["config"]["nccl_world_size"] = world
     if world == 1 and not args.no_cpu_baseline:
         line["cpu_baseline"] = cpu_baseline(args.config, g)
     return line
+
+
+def _timed_solves(args, mk, flush, stream, card_ref, before=None):
+    """Create a handle per step (untimed), optionally prepare (untimed), flush L2,
+    time mcm_solve alone with CUDA events on the solve stream; returns (ms list,
+    stats of the last solve)."""
+    import torch
+
+    ms, st = [], None
+    for i in range(args.warmup + args.steps):
+        mt = mk()
+        if before:
+            before(mt)
+        flush.fill_(i & 0xFF)
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(stream)
+        card = mt.solve_into()
+        b.record(stream)
+        b.synchronize()
+        st = mt.stats()
+        mt.close()
+        if card != card_ref:
+            raise RuntimeError(f"cardinality {card} != {card_ref}")
+        if i >= args.warmup:
+            ms.append(a.elapsed_time(b))
+    return ms, st
+
+
+def run_paper_protocol(args, g, ip, ix, ws, rm, cm, flush, stream, opts, card_ref):
+    """t_pr: the paper times the matching from a cheap
+    initial matching computed beforehand.  Per step: mcm_create + mcm_initial_matching
+    (the device greedy, R13) outside the timed region, then mcm_solve with
+    MCM_INIT_GIVEN from that M0, timed alone."""
+    m0 = []
+
+    def mk():
+        mt = pkg_matcher(ip, ix, g, ws, dict(opts, init="given"))
+        mt.solve_into = lambda: mt.solve(rm, cm)[0]
+        return mt
+
+    def before(mt):
+        m0.append(mt.initial_matching(rm, cm)[0])
+
+    ms, st = _timed_solves(args, mk, flush, stream, card_ref, before)
+    t = statistics.median(ms)
+    return {"t_pr_ms_median": t, "t_pr_ms_mean": statistics.mean(ms), "t_pr_ms_min": min(ms),
+            "edges_per_s": g.nnz / (t * 1e-3), "m0_card": m0[-1], "mm": card_ref,
+            "loops": st["loops"], "gr_count": st["gr_count"], "gr_levels": st["gr_levels"],
+            "what": "mcm_solve alone, init=given from the device cheap matching (mcm_initial_matching, untimed); "
+                    "create untimed (P:719-722)"}
+
+
+def run_paper_config(args, g, ip, ix, ws, rm, cm, flush, stream, card_ref):
+    """The paper's atomic-free G-PR: one push per column per loop
+    (no push chains, R26), complete GRs (no early stop, R22 / R28), post-GR shrink
+    only (no adaptive compaction), k = 0.7.  Solve timed alone (create
+    untimed), same graph, same L2 flush."""
+    def mk():
+        mt = pkg_matcher(ip, ix, g, ws, PAPER_OPTS)
+        mt.solve_into = lambda: mt.solve(rm, cm)[0]
+        return mt
+
+    ms, st = _timed_solves(args, mk, flush, stream, card_ref)
+    t = statistics.median(ms)
+    return {"options": PAPER_OPTS, "ms_solve_median": t, "ms_solve_mean": statistics.mean(ms),
+            "edges_per_s_solve_only": g.nnz / (t * 1e-3), "mm": card_ref,
+            "loops": st["loops"], "gr_count": st["gr_count"], "gr_levels": st["gr_levels"],
+            "pushes": st["pushes"], "blocked": st["blocked"], "guard_reactivated": st["guard_reactivated"]}
+
+
+def pkg_matcher(ip, ix, g, ws, opts):
+    import paper_conf_icpp_devecikuc13_b200 as pkg
+
+    mt = pkg.Matcher.__new__(pkg.Matcher)
+    mt_init(mt, ip, ix, g, ws, opts)
+    return mt
 
 
 def mt_init(mt, ip, ix, g, ws, opts, stream=None):
@@ -502,7 +602,7 @@ def run_batch(args, rank, world, local_rank):
         "e2e": {"value": nnz_total / (t_e2e_max * 1e-3), "unit": "edges/s",
                 "h2d_bytes_per_step": int(sum(4 * (g.m + 1 + g.nnz) for g in graphs)),
                 "d2h_bytes_per_step": int(sum(4 * (g.m + g.n) for g in graphs)), "ms_per_step": t_e2e_max},
-        "gpu_launches": args.steps * 7 * len(graphs),
+        "gpu_launches": args.steps * sum(st_["kernel_launches"] for st_ in stats),
     }
     if world == 1 and not args.no_cpu_baseline:
         line["cpu_baseline"] = cpu_baseline("C5", graphs[0])
@@ -510,25 +610,77 @@ def run_batch(args, rank, world, local_rank):
     return line
 
 
-def cpu_baseline(name, g, budget_s=20.0):
-    """The oracle's sequential PR-FIFO (k = 0.5) incl. its cheap matching,
-    single-threaded on the host: a reported baseline, not the target."""
+def host_info():
+    """nproc, the cores this process may use, the CPU model."""
+    model = None
+    try:
+        for ln in open("/proc/cpuinfo"):
+            if ln.startswith("model name"):
+                model = ln.split(":", 1)[1].strip()
+                break
+    except OSError:
+        pass
+    try:
+        allowed = sorted(os.sched_getaffinity(0))
+    except AttributeError:
+        allowed = list(range(os.cpu_count() or 1))
+    return {"nproc": os.cpu_count(), "cores_allowed": len(allowed), "cpu_model": model}, allowed
+
+
+def _pinned(fn, core, out, key):
+    """Run fn() in this thread pinned to one core (ctypes releases the GIL, so two
+    oracle calls run truly concurrently)."""
+    try:
+        os.sched_setaffinity(threading.get_native_id(), {core})
+    except (AttributeError, OSError):
+        pass
+    t0 = time.perf_counter()
+    r = fn()
+    out[key] = (time.perf_counter() - t0, r)
+
+
+def cpu_baseline(name, g, budget_s=60.0):
+    """The oracle as it stands, on the host, rank 0 at N = 1: its sequential
+    PR-FIFO (Alg. 1 + GR every 0.5(m+n) pushes, P:706-709 -- the paper's CPU
+    comparison algorithm) and its Hopcroft-Karp, both from the same host cheap
+    matching (computed once, timed separately, excluded like P:720-722), each
+    single-threaded and pinned to its own core, the two running concurrently.  A
+    reported baseline, not the target."""
     import oracle
 
+    info, allowed = host_info()
     csc = oracle.transpose(g)
-    times = []
+    t0 = time.perf_counter()
+    _, rm0, cm0 = oracle.cheap_match(g, csc)
+    t_cheap = time.perf_counter() - t0
+    init = (rm0, cm0)
+    runs = {"pr": [], "hk": []}
+    cards = set()
     t_start = time.perf_counter()
+    c_pr, c_hk = allowed[0], allowed[1 % len(allowed)]
     while True:
-        t0 = time.perf_counter()
-        oracle.cheap_match(g, csc)
-        card, _, _, _ = oracle.pr_fifo(g, k=0.5, csc=csc)
-        times.append(time.perf_counter() - t0)
-        if time.perf_counter() - t_start > budget_s * 0.5 or len(times) >= 5:
+        out = {}
+        ths = [threading.Thread(target=_pinned, args=(lambda: oracle.pr_fifo(g, k=0.5, init=init, csc=csc)[0], c_pr,
+                                                      out, "pr")),
+               threading.Thread(target=_pinned, args=(lambda: oracle.hopcroft_karp(g, init=init, csc=csc)[0], c_hk,
+                                                      out, "hk"))]
+        for th in ths:
+            th.start()
+        for th in ths:
+            th.join()
+        for k in ("pr", "hk"):
+            runs[k].append(out[k][0])
+            cards.add(out[k][1])
+        if time.perf_counter() - t_start > budget_s * 0.5 or len(runs["pr"]) >= 3:
             break
-    t = statistics.median(times)
-    return {"value": g.nnz / t, "unit": "edges/s", "cores": 1, "kind": "oracle",
-            "sample": f"full {name} graph ({g.nnz} nnz), sequential PR-FIFO + cheap matching, "
-                      f"median of {len(times)} runs ({t:.3f} s each)", "card": card}
+    t_pr, t_hk = statistics.median(runs["pr"]), statistics.median(runs["hk"])
+    if len(cards) != 1:
+        raise RuntimeError(f"oracle disagreement {cards}")
+    return {"value": g.nnz / t_pr, "unit": "edges/s", "cores": 2 if c_pr != c_hk else 1, "kind": "oracle",
+            "sample": f"full {name} graph ({g.nnz} nnz), {len(runs['pr'])} run(s): PR-FIFO (value) and Hopcroft-Karp, "
+                      f"single-threaded, concurrently on cores {c_pr} / {c_hk}, both from the host cheap matching",
+            "pr_fifo_ms": t_pr * 1e3, "hopcroft_karp_ms": t_hk * 1e3, "hk_edges_per_s": g.nnz / t_hk,
+            "cheap_match_ms": t_cheap * 1e3, "m0_card": int((rm0 >= 0).sum()), "card": cards.pop(), **info}
 
 
 def run_reference(args, rank):
@@ -536,10 +688,13 @@ def run_reference(args, rank):
         return None
     g = _graph(args.config, 0)
     times = []
-    cb = None
+    import oracle
+
+    info, allowed = host_info()
+    csc = oracle.transpose(g)
     for i in range(args.warmup + args.steps):
         t0 = time.perf_counter()
-        cb = cpu_baseline(args.config, g, budget_s=0.0)  # one PR-FIFO run per step
+        oracle.pr_fifo(g, k=0.5, csc=csc)  # incl. the cheap matching it starts from
         dt = time.perf_counter() - t0
         if i >= args.warmup:
             times.append(dt)
@@ -552,7 +707,7 @@ def run_reference(args, rank):
         "config": {"workload": f"{args.config}: {CONFIG_DESC[args.config]}", "m": g.m, "n": g.n, "nnz": g.nnz},
         "cpu_baseline": {"value": v, "unit": "edges/s", "cores": 1, "kind": "oracle",
                          "sample": f"full {args.config} graph per step: cheap matching + sequential PR-FIFO "
-                                   f"(k=0.5), single core"},
+                                   f"(k=0.5), single core", **info},
         "e2e": {"value": v, "unit": "edges/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
 
@@ -562,7 +717,7 @@ def main():
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=20)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--config", default="C2", choices=sorted(CONFIG_DESC))
+    ap.add_argument("--config", default="C4", choices=sorted(CONFIG_DESC))
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--k", type=float, default=0.4)
     ap.add_argument("--no-cpu-baseline", action="store_true")

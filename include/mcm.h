@@ -30,9 +30,10 @@
  * The handle itself is a small host object.
  *
  * Streams.  Every call enqueues its device work on the given stream; nothing
- * touches the legacy default stream or synchronises the device.  mcm_create and
- * mcm_solve synchronise `stream` once each (to return an error code / the
- * cardinality).  A handle is bound to the device current at mcm_create; calling
+ * touches the legacy default stream or synchronises the device.  mcm_create
+ * synchronises `stream` twice (the validation result, then the end of the
+ * transpose); mcm_solve and the other device entry points once (to return their
+ * result).  A handle is bound to the device current at mcm_create; calling
  * it with another device current returns MCM_EDEVICE.  One handle per host
  * thread (handles are not thread-safe).  After MCM_ECUDA the handle is poisoned:
  * every later call returns MCM_ECUDA.
@@ -65,8 +66,13 @@ enum {
 enum { MCM_GR_ADAPTIVE = 0, MCM_GR_FIXED = 1 };
 
 /* Initial matching: cheap greedy on the device (reading R13), the
- * caller's matching in rmatch/cmatch (must be a valid matching whose two arrays
- * are mutually consistent), or empty. */
+ * caller's matching in rmatch/cmatch, or empty.  GIVEN: every rmatch[u] must be
+ * -1 or a column (< n) and every cmatch[v] -1 or a row (< m), else mcm_solve
+ * returns MCM_EINVAL (checked on the device before any phase runs).  Pairs that
+ * do not point back at each other are tolerated, with the paper's conventions: a
+ * column whose row does not point back is unmatched (Alg. 6 l.3, reading R1); a
+ * row whose column does not point back is repaired before the exactness guard's
+ * GR (reading R27).  The pairs are not checked to be edges. */
 enum { MCM_INIT_GREEDY = 0, MCM_INIT_GIVEN = 1, MCM_INIT_EMPTY = 2 };
 
 typedef struct {
@@ -118,7 +124,7 @@ typedef struct {
   int32_t variant;      /* 0 (default): G-PR (Alg. 7, active-column worklist);
                            1: G-PR-First (Alg. 3 + Alg. 6: every column
                            tested every loop; the Fig. 1 ablation) */
-  int32_t tail_chain;   /* single-CTA tail with at most 16 active columns: each column's warp
+  int32_t tail_chain;   /* single-CTA tail with at most 32 active columns: each column's lanes
                            runs a chain of double pushes (the displaced column is pushed next
                            by the same warp, its row claimed by CAS) instead of one push per
                            loop -- a build addition (R26); 0 = the paper's one push
@@ -157,7 +163,12 @@ typedef struct {
   int64_t gr_edges;          /* adjacency entries read by all GR levels */
   int64_t gr_cols;           /* columns labelled by all GRs */
   int64_t greedy_edges;      /* adjacency entries read by the greedy initial matching */
-  int64_t rows_repaired;     /* stale rows (mate not pointing back) made unmatched before the guard GR (R27) */
+  int64_t rows_repaired;     /* stale rows (mate not pointing back) re-attached or made unmatched before
+                                the guard GR (R27) */
+  int64_t tail_gr_levels;    /* GR levels run by the single-CTA tail (frontier in shared memory) */
+  int64_t debug_violations;  /* consistency violations found by the debug checks (env MCM_DEBUG=1) */
+  int64_t kernel_launches;   /* kernels launched by this handle's mcm_create plus by the last call (counted
+                                at the launch sites: the create's setup kernels + one persistent kernel) */
   double ms_init;            /* device time: initial matching + worklist build */
   double ms_gr;              /* device time in global relabels */
   double ms_loop;            /* device time in fix + push steps */
@@ -202,15 +213,59 @@ int64_t mcm_match_host(const int32_t *indptr, const int32_t *indices, int32_t m,
                        void *workspace, size_t ws_bytes, mcm_stream_t stream, const mcm_options_t *o,
                        int32_t *rmatch, int32_t *cmatch, mcm_stats_t *stats);
 
-/* Global relabel (Alg. 4/5) of a given matching: rmatch (m) and cmatch
- * (n) are DEVICE inputs with the paper's mu conventions (column entries may be
- * stale or -2; rows are authoritative); writes psi_row (m) and psi_col
- * (n) (DEVICE) = exact alternating BFS distance from the unmatched rows, m+n when
- * unreached.  Returns maxLevel = (deepest row level) + 2 (Alg. 4's final cLevel),
- * or a negative error code.  *reached_free (may be NULL) = number of columns that
- * are not matched but got a finite label (> 0 iff an augmenting path exists). */
+/* Global relabel (Alg. 4/5) of a given matching, run exactly as a solve
+ * runs its GRs under the handle's options: grid BFS levels, single-CTA tail levels
+ * with the frontier in shared memory (tail_max > 0 and frontiers of at most tail_f
+ * rows, handed back to the grid above it), bottom-up levels (bu_div), and the
+ * early stop of gr_early / gr_target / gr_target_min (R22 / R28).
+ * rmatch (m) and cmatch (n) are DEVICE inputs with the paper's mu conventions
+ * (column entries may be stale or -2; rows are authoritative; ranges as
+ * for MCM_INIT_GIVEN, cmatch may also hold -2, else MCM_EINVAL).  Writes psi_row (m)
+ * and psi_col (n) (DEVICE): the exact alternating BFS distance from the unmatched
+ * rows for every vertex the BFS labelled; a vertex it did not reach gets m+n after
+ * a complete GR, and the lower bound floor_row / floor_col after an early stop.
+ * Returns maxLevel as GETITERGR uses it ((deepest row level) + 2, Alg. 4's final
+ * cLevel; after an early stop at row level l: l + 4), or a negative error code.
+ * info (may be NULL) receives 4 values: [0] the number of columns that are not
+ * matched but got a finite label (> 0 iff an augmenting path exists, after a
+ * complete GR), [1] floor_row, [2] floor_col (m+n after a complete GR), [3] the
+ * BFS levels the single-CTA tail ran. */
 int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,
-                           int32_t *psi_row, int32_t *psi_col, int64_t *reached_free);
+                           int32_t *psi_row, int32_t *psi_col, int64_t *info);
+
+/* The cheap initial matching alone (reading R13: every column
+ * claims the first free row of Gamma(v) by CAS -- the phase a default mcm_solve
+ * starts with).  Writes rmatch (m) / cmatch (n) (DEVICE) = M0, a valid maximal
+ * matching, and returns |M0| or a negative error code.  Used for the paper's timing
+ * protocol (the cheap matching excluded from the timed solve: feed M0 to
+ * mcm_solve with MCM_INIT_GIVEN) and to test M0 on its own. */
+int64_t mcm_initial_matching(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t *cmatch);
+
+/* ONE phase of the solve kernel on a caller-given state (test and inspection
+ * entry point: the code a solve runs, not a re-implementation).
+ *   unit  MCM_UNIT_FIX         G-PR-INITKRNL (Alg. 8): rollback of lost
+ *                              pushes, iA marks; returns the active-slot count
+ *         MCM_UNIT_SHRINK      G-PR-SHRKRNL: the same with the surviving
+ *                              slots compacted in slot order; returns the new length
+ *         MCM_UNIT_PUSH        G-PR-PUSHKRNL (Alg. 9; no push chains);
+ *                              returns 0
+ *         MCM_UNIT_FIXMATCHING FIXMATCHING: mu_col <- the output
+ *                              convention (reading R15); returns |M|
+ *   where MCM_WHERE_GRID (every CTA, the phase code of a wide loop) or
+ *         MCM_WHERE_TAIL (CTA 0 alone with the worklist in shared memory when it
+ *         fits, as the solve's tail mode runs it; the tail fix step always compacts,
+ *         so FIX there behaves as SHRINK).  FIXMATCHING always runs on the grid.
+ *   loop  the loop counter (iA marks, Alg. 9 l.13), 0 <= loop < 2^31
+ *   len   worklist slots, 0 <= len <= n
+ * In/out DEVICE int32 arrays: mu_row (m, -1 or a column), mu_col (n, -2, -1 or a
+ * row), psi_row (m) and psi_col (n) (labels; < 0 or >= m+n mean m+n on input),
+ * iA (n), Ac (len), Ap (len).  Out-of-range entries return MCM_EINVAL.  The
+ * phase's statistics (pushes, blocked, dead, slots) are in mcm_get_stats. */
+enum { MCM_UNIT_FIX = 0, MCM_UNIT_SHRINK = 1, MCM_UNIT_PUSH = 2, MCM_UNIT_FIXMATCHING = 3 };
+enum { MCM_WHERE_GRID = 0, MCM_WHERE_TAIL = 1 };
+int64_t mcm_unit_step(mcm_handle_t h, mcm_stream_t stream, int32_t unit, int32_t where, int64_t loop, int32_t len,
+                      int32_t *mu_row, int32_t *mu_col, int32_t *psi_row, int32_t *psi_col, int32_t *iA, int32_t *Ac,
+                      int32_t *Ap);
 
 /* Gap relabelling (reading R14) of given labels, in place: psi_row (m)
  * and psi_col (n) are DEVICE int32 labels (values >= m+n, or < 0, mean infinite).

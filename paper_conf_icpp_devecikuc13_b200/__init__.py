@@ -11,6 +11,7 @@ Names follow include/mcm.h:
 
 * :func:`mcm_default_options`, :func:`mcm_workspace_bytes`
 * :class:`Matcher` -- ``mcm_create`` / ``mcm_solve`` / ``mcm_global_relabel`` /
+  ``mcm_initial_matching`` / ``mcm_unit_step`` / ``mcm_gap_relabel`` /
   ``mcm_set_options`` / ``mcm_get_stats`` / ``mcm_destroy`` on one graph
 * :func:`solve` -- create + solve in one call: ``(card, rmatch, cmatch)``
 * :func:`match_host` -- ``mcm_match_host``: host CSR in, host matching out (the
@@ -30,6 +31,8 @@ LIB_PATH = os.environ.get("MCM_LIB") or os.path.join(_HERE, "libmcm.so")  # MCM_
 MCM_OK, MCM_EINVAL, MCM_ECUDA, MCM_ENOMEM, MCM_EDEVICE, MCM_ENOCONV, MCM_EINTERNAL = 0, -1, -2, -3, -4, -5, -6
 MCM_GR_ADAPTIVE, MCM_GR_FIXED = 0, 1
 MCM_INIT_GREEDY, MCM_INIT_GIVEN, MCM_INIT_EMPTY = 0, 1, 2
+MCM_UNIT_FIX, MCM_UNIT_SHRINK, MCM_UNIT_PUSH, MCM_UNIT_FIXMATCHING = 0, 1, 2, 3
+MCM_WHERE_GRID, MCM_WHERE_TAIL = 0, 1
 
 
 class Options(ctypes.Structure):
@@ -69,7 +72,7 @@ class Stats(ctypes.Structure):
     _fields_ = [(f, ctypes.c_int64) for f in (
         "loops", "gr_count", "gr_levels", "pushes", "blocked", "dead", "edges_scanned", "slots", "shrinks", "gaps",
         "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers", "gr_rows", "gr_edges",
-        "gr_cols", "greedy_edges", "rows_repaired")] + [
+        "gr_cols", "greedy_edges", "rows_repaired", "tail_gr_levels", "debug_violations", "kernel_launches")] + [
         (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
         ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
 
@@ -105,8 +108,12 @@ def lib():
         L.mcm_solve.restype = i64
         L.mcm_match_host.argtypes = [vp, vp, i32, i32, i64, vp, sz, vp, P(Options), vp, vp, P(Stats)]
         L.mcm_match_host.restype = i64
-        L.mcm_global_relabel.argtypes = [vp, vp, vp, vp, vp, vp, P(i64)]
+        L.mcm_global_relabel.argtypes = [vp, vp, vp, vp, vp, vp, vp]
         L.mcm_global_relabel.restype = i64
+        L.mcm_initial_matching.argtypes = [vp, vp, vp, vp]
+        L.mcm_initial_matching.restype = i64
+        L.mcm_unit_step.argtypes = [vp, vp, i32, i32, i64, i32, vp, vp, vp, vp, vp, vp, vp]
+        L.mcm_unit_step.restype = i64
         L.mcm_gap_relabel.argtypes = [vp, vp, vp, vp]
         L.mcm_gap_relabel.restype = i64
         L.mcm_set_options.argtypes = [vp, P(Options)]
@@ -155,8 +162,14 @@ def _torch():
 
 
 def _stream_ptr(stream):
+    """The stream the library enqueues on.  A stream other than the current one is
+    first ordered after the current stream, where the caller's inputs, outputs and
+    workspace were produced / allocated (torch's caching allocator is stream-ordered)."""
     torch = _torch()
-    s = stream if stream is not None else torch.cuda.current_stream()
+    cur = torch.cuda.current_stream()
+    s = stream if stream is not None else cur
+    if s != cur:
+        s.wait_stream(cur)
     return ctypes.c_void_p(s.cuda_stream)
 
 
@@ -218,19 +231,53 @@ class Matcher:
             raise MCMError(int(card), "mcm_solve")
         return int(card), rmatch, cmatch
 
-    def global_relabel(self, rmatch, cmatch, stream=None):
-        """mcm_global_relabel -> (max_level, psi_row, psi_col, reached_free)."""
+    def global_relabel(self, rmatch, cmatch, stream=None, info=False):
+        """mcm_global_relabel -> (max_level, psi_row, psi_col, reached_free), plus
+        dict(floor_row, floor_col, tail_levels) when info=True."""
         torch = _torch()
         pr = torch.empty(self.m, dtype=torch.int32, device=self.device)
         pc = torch.empty(self.n, dtype=torch.int32, device=self.device)
-        rf = ctypes.c_int64(0)
+        inf = (ctypes.c_int64 * 4)()
         with torch.cuda.device(self.device):
             ml = lib().mcm_global_relabel(self._h, _stream_ptr(stream), _dev_i32(rmatch, "rmatch", self.m),
                                           _dev_i32(cmatch, "cmatch", self.n), _dev_i32(pr, "psi_row", self.m),
-                                          _dev_i32(pc, "psi_col", self.n), ctypes.byref(rf))
+                                          _dev_i32(pc, "psi_col", self.n), inf)
         if ml < 0:
             raise MCMError(int(ml), "mcm_global_relabel")
-        return int(ml), pr, pc, int(rf.value)
+        if info:
+            return int(ml), pr, pc, int(inf[0]), dict(floor_row=int(inf[1]), floor_col=int(inf[2]), tail_levels=int(inf[3]))
+        return int(ml), pr, pc, int(inf[0])
+
+    def initial_matching(self, rmatch=None, cmatch=None, stream=None):
+        """mcm_initial_matching -> (|M0|, rmatch, cmatch): the device cheap matching alone."""
+        torch = _torch()
+        if rmatch is None:
+            rmatch = torch.empty(self.m, dtype=torch.int32, device=self.device)
+        if cmatch is None:
+            cmatch = torch.empty(self.n, dtype=torch.int32, device=self.device)
+        with torch.cuda.device(self.device):
+            c = lib().mcm_initial_matching(self._h, _stream_ptr(stream), _dev_i32(rmatch, "rmatch", self.m),
+                                           _dev_i32(cmatch, "cmatch", self.n))
+        if c < 0:
+            raise MCMError(int(c), "mcm_initial_matching")
+        return int(c), rmatch, cmatch
+
+    def unit_step(self, unit, where, loop, mu_row, mu_col, psi_row, psi_col, iA, Ac, Ap, stream=None):
+        """mcm_unit_step on the given CUDA int32 tensors (updated in place) -> the
+        phase's result (see include/mcm.h)."""
+        torch = _torch()
+        unit = {"fix": MCM_UNIT_FIX, "shrink": MCM_UNIT_SHRINK, "push": MCM_UNIT_PUSH,
+                "fixmatching": MCM_UNIT_FIXMATCHING}.get(unit, unit)
+        where = {"grid": MCM_WHERE_GRID, "tail": MCM_WHERE_TAIL}.get(where, where)
+        ln = int(Ac.numel())
+        with torch.cuda.device(self.device):
+            r = lib().mcm_unit_step(self._h, _stream_ptr(stream), unit, where, int(loop), ln,
+                                    _dev_i32(mu_row, "mu_row", self.m), _dev_i32(mu_col, "mu_col", self.n),
+                                    _dev_i32(psi_row, "psi_row", self.m), _dev_i32(psi_col, "psi_col", self.n),
+                                    _dev_i32(iA, "iA", self.n), _dev_i32(Ac, "Ac", ln), _dev_i32(Ap, "Ap", ln))
+        if r < 0:
+            raise MCMError(int(r), "mcm_unit_step")
+        return int(r)
 
     def gap_relabel(self, psi_row, psi_col, stream=None):
         """mcm_gap_relabel on copies of the given labels -> (gap, psi_row', psi_col')."""

@@ -201,6 +201,7 @@ struct mcm_ctx {
   bool poisoned = false;
   mcm_stats_t stats;
   double ms_setup = 0;
+  int create_launches = 0;
   Ctrl host_ctrl;
 };
 
@@ -320,6 +321,7 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
   CK(cudaMemsetAsync(cnt, 0, sizeof(int) * ((size_t)n + 1), st));
   int vb = (int)std::min<long long>(std::max<long long>((nnz + 1023) / 1024, (m + 255) / 256 + 1), 148 * 8);
   k_ingest<<<vb, 256, 0, st>>>(vp, vi, m, n, nnz, rptr, radj, cnt, err, from_host ? 0 : 1);
+  int nlaunch = 1;  // kernels this create launched (mcm_stats_t.kernel_launches)
   CK(cudaGetLastError());
   int herr = 0;
   CK(cudaMemcpyAsync(&herr, err, sizeof(int), cudaMemcpyDeviceToHost, st));
@@ -336,6 +338,7 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
   k_scan_sums<<<nb, 512, 0, st>>>(cnt, n, bsum);
   k_scan_bsum<<<1, 1024, 0, st>>>(bsum, nb);
   k_scan_apply<<<nb, 1024, 0, st>>>(cnt, n, bsum, cptr, n);
+  nlaunch += 3;
   CK(cudaGetLastError());
   if (n == 0) CK(cudaMemsetAsync(cptr, 0, sizeof(int), st));
   CK(cudaMemcpyAsync(cursor, cptr, sizeof(int) * ((size_t)n + 1), cudaMemcpyDeviceToDevice, st));
@@ -343,9 +346,11 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
     long long warps = (nnz + 32 * SC_K - 1) / (32 * SC_K);
     int sb = (int)std::min<long long>((warps + 7) / 8, 148 * 32);
     k_scatter<<<sb, 256, 0, st>>>(rptr, radj, m, nnz, cursor, cadj);
+    nlaunch++;
     CK(cudaGetLastError());
     if (h->opt.sort_csc) {
       k_sort_segments<<<(n + 255) / 256, 256, 0, st>>>(cptr, cadj, n);
+      nlaunch++;
       CK(cudaGetLastError());
     }
   }
@@ -353,6 +358,7 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
   CK(cudaStreamSynchronize(st));
   h->ms_setup = std::chrono::duration<double, std::milli>(std::chrono::steady_clock::now() - t0).count();
   memset(&h->stats, 0, sizeof(h->stats));
+  h->create_launches = nlaunch;
   *out = guard.release();
   return MCM_OK;
 }
@@ -362,10 +368,20 @@ int mcm_create(const int32_t *indptr, const int32_t *indices, int32_t m, int32_t
   return create_impl(indptr, indices, m, n, nnz, workspace, ws_bytes, stream, o, out, false);
 }
 
+// MODE_UNIT: the phase to run, the caller's label arrays, and the device copies
+// of the caller's iA / Ac / Ap into the workspace (before the kernel) and back
+// (after it)
+struct UnitArgs {
+  int what, where, len;
+  long long loop;
+  int32_t *psi_r, *psi_c, *iA, *Ac, *Ap;
+};
+
 // host_r / host_c (optional): HOST buffers the outputs are copied into before the
 // single synchronisation
 static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin, const int32_t *cin, int32_t *out_r,
-                      int32_t *out_c, int32_t *host_r = nullptr, int32_t *host_c = nullptr) {
+                      int32_t *out_c, int32_t *host_r = nullptr, int32_t *host_c = nullptr,
+                      const UnitArgs *ua = nullptr) {
   if (h->poisoned) return MCM_ECUDA;
   int dev = -1;
   CK(cudaGetDevice(&dev));
@@ -410,9 +426,10 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_chain = o.tail_chain;
   // worklists of at most this many slots run as push chains (lanes per slot from the
   // count); MCM_CHAIN_SLOTS: analysis knob
-  p.chain_slots = getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 32;
+  // (analysis knobs, clamped: 0..TW slots; a divisor of at least 1)
+  p.chain_slots = std::min(std::max(getenv("MCM_CHAIN_SLOTS") ? atoi(getenv("MCM_CHAIN_SLOTS")) : 32, 0), TW);
   p.grid_chain = o.grid_chain;
-  p.grid_chain_div = getenv("MCM_GRID_CHAIN_DIV") ? atoi(getenv("MCM_GRID_CHAIN_DIV")) : 2;
+  p.grid_chain_div = std::max(getenv("MCM_GRID_CHAIN_DIV") ? atoi(getenv("MCM_GRID_CHAIN_DIV")) : 2, 1);
   p.bu_div = o.bu_div;
   p.scan_rot = o.serial ? 0 : o.scan_rot;
   if (o.variant == 1) {  // G-PR-First: no worklist, so no tail group either
@@ -429,7 +446,16 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
   p.rmatch_in = rin; p.cmatch_in = cin; p.rmatch_out = out_r; p.cmatch_out = out_c;
-  int C = o.tail_ctas;
+  if (ua) {
+    p.unit_what = ua->what; p.unit_where = ua->where; p.unit_len = ua->len; p.unit_loop = ua->loop;
+    p.psi_row_io = ua->psi_r; p.psi_col_io = ua->psi_c;
+    if (h->n) CK(cudaMemcpyAsync(p.iA, ua->iA, sizeof(int) * (size_t)h->n, cudaMemcpyDeviceToDevice, st));
+    if (ua->len) {
+      CK(cudaMemcpyAsync(p.wl0, ua->Ac, sizeof(int) * (size_t)ua->len, cudaMemcpyDeviceToDevice, st));
+      CK(cudaMemcpyAsync(p.wl1, ua->Ap, sizeof(int) * (size_t)ua->len, cudaMemcpyDeviceToDevice, st));
+    }
+  }
+  int C = mode == MODE_UNIT ? 1 : o.tail_ctas;  // a unit's tail is CTA 0 alone
   // the lean production instance unless a feature only the full one carries is on
   // (a cluster tail group spans several SMs' L1s: it needs gpu-scope vertex state)
   void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1)
@@ -466,6 +492,13 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = sizeof(Smem); cfg.stream = st;
   cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
   CK(cudaLaunchKernelEx(&cfg, kern, p));
+  if (ua) {
+    if (h->n) CK(cudaMemcpyAsync(ua->iA, p.iA, sizeof(int) * (size_t)h->n, cudaMemcpyDeviceToDevice, st));
+    if (ua->len) {
+      CK(cudaMemcpyAsync(ua->Ac, p.wl0, sizeof(int) * (size_t)ua->len, cudaMemcpyDeviceToDevice, st));
+      CK(cudaMemcpyAsync(ua->Ap, p.wl1, sizeof(int) * (size_t)ua->len, cudaMemcpyDeviceToDevice, st));
+    }
+  }
   if (host_r && h->m) CK(cudaMemcpyAsync(host_r, out_r, sizeof(int32_t) * (size_t)h->m, cudaMemcpyDeviceToHost, st));
   if (host_c && h->n) CK(cudaMemcpyAsync(host_c, out_c, sizeof(int32_t) * (size_t)h->n, cudaMemcpyDeviceToHost, st));
   CK(cudaMemcpyAsync(&h->host_ctrl, p.ctrl, sizeof(Ctrl), cudaMemcpyDeviceToHost, st));
@@ -479,7 +512,9 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   s.shrinks = x[ST_SHRINKS]; s.gaps = x[ST_GAPS]; s.guard_reactivated = x[ST_GUARD]; s.fixed_cols = x[ST_FIXED];
   s.init_card = x[ST_INITCARD]; s.card = x[ST_CARD]; s.tail_loops = x[ST_TAILLOOPS]; s.grid_barriers = x[ST_BARRIERS];
   s.gr_rows = x[ST_GR_ROWS]; s.gr_edges = x[ST_GR_EDGES]; s.gr_cols = x[ST_GR_COLS];
-  s.greedy_edges = x[ST_GREEDY_EDGES]; s.rows_repaired = x[ST_REPAIRED];
+  s.greedy_edges = x[ST_GREEDY_EDGES]; s.rows_repaired = x[ST_REPAIRED]; s.tail_gr_levels = x[ST_TAIL_LEVELS];
+  s.debug_violations = c.dbg[0];
+  s.kernel_launches = h->create_launches + 1;  // the create's kernels + this call's one persistent kernel
   s.ms_init = x[ST_NS_INIT] * 1e-6; s.ms_gr = x[ST_NS_GR] * 1e-6; s.ms_loop = x[ST_NS_LOOP] * 1e-6;
   s.ms_total = x[ST_NS_TOTAL] * 1e-6; s.ms_setup = h->ms_setup; s.grid_ctas = grid; s.threads_per_cta = NT;
   if (p.debug && c.dbg[0])
@@ -493,7 +528,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     if (f) { fwrite(buf.data(), sizeof(long long), buf.size(), f); fclose(f); }
   }
   if (c.err) return c.err;
-  if (mode == MODE_RELABEL || mode == MODE_GAP) return x[ST_MAXLEVEL];
+  if (mode == MODE_RELABEL || mode == MODE_GAP || mode == MODE_UNIT) return x[ST_MAXLEVEL];
   return x[ST_CARD];
 }
 
@@ -519,12 +554,33 @@ int64_t mcm_match_host(const int32_t *indptr, const int32_t *indices, int32_t m,
 }
 
 int64_t mcm_global_relabel(mcm_handle_t h, mcm_stream_t stream, const int32_t *rmatch, const int32_t *cmatch,
-                           int32_t *psi_row, int32_t *psi_col, int64_t *reached_free) {
+                           int32_t *psi_row, int32_t *psi_col, int64_t *info) {
   if (!h) return MCM_EINVAL;
   if ((h->m > 0 && (!rmatch || !psi_row)) || (h->n > 0 && (!cmatch || !psi_col))) return MCM_EINVAL;
   int64_t r = launch(h, (cudaStream_t)stream, MODE_RELABEL, rmatch, cmatch, psi_row, psi_col);
-  if (r >= 0 && reached_free) *reached_free = h->host_ctrl.stat[ST_REACHED_FREE];
+  if (r >= 0 && info) {
+    const long long *x = h->host_ctrl.stat;
+    info[0] = x[ST_REACHED_FREE]; info[1] = x[ST_FLOOR_R]; info[2] = x[ST_FLOOR_C]; info[3] = x[ST_TAIL_LEVELS];
+  }
   return r;
+}
+
+int64_t mcm_initial_matching(mcm_handle_t h, mcm_stream_t stream, int32_t *rmatch, int32_t *cmatch) {
+  if (!h) return MCM_EINVAL;
+  if ((h->m > 0 && !rmatch) || (h->n > 0 && !cmatch)) return MCM_EINVAL;
+  return launch(h, (cudaStream_t)stream, MODE_INIT, nullptr, nullptr, rmatch, cmatch);
+}
+
+int64_t mcm_unit_step(mcm_handle_t h, mcm_stream_t stream, int32_t unit, int32_t where, int64_t loop, int32_t len,
+                      int32_t *mu_row, int32_t *mu_col, int32_t *psi_row, int32_t *psi_col, int32_t *iA, int32_t *Ac,
+                      int32_t *Ap) {
+  if (!h || unit < MCM_UNIT_FIX || unit > MCM_UNIT_FIXMATCHING || (where != MCM_WHERE_GRID && where != MCM_WHERE_TAIL))
+    return MCM_EINVAL;
+  if (loop < 0 || loop > 0x7fffffffLL || len < 0 || len > h->n) return MCM_EINVAL;
+  if ((h->m > 0 && (!mu_row || !psi_row)) || (h->n > 0 && (!mu_col || !psi_col || !iA)) || (len > 0 && (!Ac || !Ap)))
+    return MCM_EINVAL;
+  UnitArgs ua{unit, where, len, loop, psi_row, psi_col, iA, Ac, Ap};
+  return launch(h, (cudaStream_t)stream, MODE_UNIT, mu_row, mu_col, mu_row, mu_col, nullptr, nullptr, &ua);
 }
 
 int64_t mcm_gap_relabel(mcm_handle_t h, mcm_stream_t stream, int32_t *psi_row, int32_t *psi_col) {

@@ -55,36 +55,19 @@ __device__ __forceinline__ long long ld_rlx(const long long *p) {
   asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
   return v;
 }
-// Vertex-state accessors with a compile-time scope.  CTA scope may be served by
-// the SM's L1 (a dependent miss costs ~140 ns instead of 175-230 ns for the strong
-// gpu-scope load, a hit after this SM's own store ~30 ns instead of ~165 ns);
-// every grid barrier invalidates L1 (its __threadfence emits CCTL.IVALL), so a
-// phase always starts from L2's values and a racy read inside a phase may at
-// most be stale -- the paper's execution model (reading R17).
-template <bool CTA>
-__device__ __forceinline__ u64 ldv(const u64 *p) {
-  u64 v;
-  if (CTA) asm volatile("ld.relaxed.cta.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
-  else asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
-  return v;
-}
-template <bool CTA>
-__device__ __forceinline__ void stv(u64 *p, u64 v) {
-  if (CTA) asm volatile("st.relaxed.cta.global.b64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
-  else asm volatile("st.relaxed.gpu.global.b64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
-}
-template <bool CTA>
-__device__ __forceinline__ int ldv(const int *p) {
-  int v;
-  if (CTA) asm volatile("ld.relaxed.cta.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
-  else asm volatile("ld.relaxed.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
-  return v;
-}
-template <bool CTA>
-__device__ __forceinline__ void stv(int *p, int v) {
-  if (CTA) asm volatile("st.relaxed.cta.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
-  else asm volatile("st.relaxed.gpu.global.b32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
-}
+// Vertex-state accessors (reading R17).  Every access to a racy vertex-state word
+// (rowst / colst / iA) is a relaxed access at GPU scope: any two of them, from
+// any two CTAs, are morally strong, so the PTX memory model gives each aligned
+// 32- or 64-bit access single-copy atomicity (a reader never sees half of one
+// packed {mu, psi} store and half of another) and the racy pushes of the paper
+// are data-race free in the model's sense.  A CTA-scope (L1-
+// cacheable) variant was measured in round 2 against this one on C2-C5
+// (tools/ab_scope.sh, profiles/r02_scope_ab.txt): every median within the
+// run-to-run spread, so the kernel keeps only the GPU-scope accessors.
+__device__ __forceinline__ u64 ldv(const u64 *p) { return ld_rlx(p); }
+__device__ __forceinline__ void stv(u64 *p, u64 v) { st_rlx(p, v); }
+__device__ __forceinline__ int ldv(const int *p) { return ld_rlx(p); }
+__device__ __forceinline__ void stv(int *p, int v) { st_rlx(p, v); }
 __device__ __forceinline__ u32 ld_acq(const u32 *p) {
   u32 v;
   asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");

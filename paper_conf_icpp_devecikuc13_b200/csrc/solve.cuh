@@ -38,16 +38,18 @@ constexpr int MAXHUGE = 32;      // CTA-wide push list per tile
 constexpr int HUGE_CTA = 4;      // at most this many per tile: one CTA-wide scan each; more: a warp each ...
 constexpr int HUGE_WARP = 8192;  // ... unless longer than this
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
-constexpr int SPLIT = 1024;
-constexpr int CHAIN_SLOTS = 128; // tail push chains (R26) for worklists of at most this many slots      // GR: a frontier row's adjacency is split into ranges of at most this many
+constexpr int SPLIT = 1024;      // GR: a frontier row's adjacency is split into ranges of at most this many
 
-enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2 };
+enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2, MODE_UNIT = 3, MODE_INIT = 4 };
+// mcm_unit_step: one phase of the solve on a given state (include/mcm.h)
+enum { UNIT_FIX = 0, UNIT_SHRINK = 1, UNIT_PUSH = 2, UNIT_FIXMATCHING = 3 };
 
 // statistics slots (Ctrl::stat)
 enum {
   ST_LOOPS, ST_GRS, ST_LEVELS, ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_SHRINKS, ST_GAPS,
   ST_GUARD, ST_FIXED, ST_INITCARD, ST_CARD, ST_TAILLOOPS, ST_BARRIERS, ST_NS_INIT, ST_NS_GR, ST_NS_LOOP,
-  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_REPAIRED, ST_NSTAT = 32
+  ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_REPAIRED,
+  ST_FLOOR_R, ST_FLOOR_C, ST_TAIL_LEVELS, ST_NSTAT = 32
 };
 
 struct Ctrl {
@@ -99,6 +101,11 @@ struct Params {
   // I/O
   const int *rmatch_in, *cmatch_in;
   int *rmatch_out, *cmatch_out;  // solve: matching; relabel: psi_row / psi_col
+  // MODE_UNIT: labels in / out, and the phase to run (Ac / Ap / iA are copied into
+  // wl0 / wl1 / iA by the host)
+  int *psi_row_io, *psi_col_io;
+  int unit_what, unit_where, unit_len;
+  long long unit_loop;
 };
 
 // per-CTA statistics accumulators (Smem::st), flushed at every barrier from
@@ -107,7 +114,7 @@ enum { SS_PUSH, SS_BLOCK, SS_DEAD, SS_SCAN, SS_SLOTS, SS_FREE, SS_GRROWS, SS_GRE
 // control-loop statistics and the phase-trace cursor: kept by the lead thread
 // (block 0, thread 0) only, in shared memory, so they hold no registers
 struct LeadStats {
-  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar, repaired;
+  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar, repaired, tail_levels;
   int tn, ttag, tsz, pad;
 };
 struct Smem;
@@ -150,19 +157,18 @@ __device__ __forceinline__ u64 tnow() { return (threadIdx.x == 0 && blockIdx.x =
 // (serial mode, G-PR-First, debug checks, gap relabelling, the label-only modes)
 // live in a second instance, so they cost the hot kernel no code size (its
 // instruction footprint is on the critical path of every short phase).
-enum { F_SERIAL = 1, F_FIRST = 2, F_DEBUG = 4, F_GAP = 8, F_AUX = 16, F_BU = 32, F_L1 = 64 };
-constexpr int F_FAST = F_BU | F_L1;  // F_L1: CTA-scope vertex state (single-CTA tail only)
+enum { F_SERIAL = 1, F_FIRST = 2, F_DEBUG = 4, F_GAP = 8, F_AUX = 16, F_BU = 32 };
+constexpr int F_FAST = F_BU;
 constexpr int F_ALL = F_SERIAL | F_FIRST | F_DEBUG | F_GAP | F_AUX | F_BU;
 
 template <int F>
 struct Solver {
   const Params &p;
-  // vertex state (rowst, colst, iA) scope: CTA (L1-cacheable) in the lean kernel
-  static constexpr bool VCTA = (F & F_L1) != 0;
-  __device__ __forceinline__ static u64 vld(const u64 *a) { return ldv<VCTA>(a); }
-  __device__ __forceinline__ static int vld(const int *a) { return ldv<VCTA>(a); }
-  __device__ __forceinline__ static void vst(u64 *a, u64 v) { stv<VCTA>(a, v); }
-  __device__ __forceinline__ static void vst(int *a, int v) { stv<VCTA>(a, v); }
+  // vertex state (rowst, colst, iA): relaxed GPU-scope accesses (device.cuh, R17)
+  __device__ __forceinline__ static u64 vld(const u64 *a) { return ldv(a); }
+  __device__ __forceinline__ static int vld(const int *a) { return ldv(a); }
+  __device__ __forceinline__ static void vst(u64 *a, u64 v) { stv(a, v); }
+  __device__ __forceinline__ static void vst(int *a, int v) { stv(a, v); }
   // the dynamic shared block, named through a namespace-scope extern __shared__
   // array so every access compiles to a shared-space instruction (a Smem& member
   // made the staging atomics generic ATOM.E)
@@ -434,9 +440,10 @@ struct Solver {
   }
 
   // ---------------------------------------------------------------- init
-  // Vertex state from the initial matching (GIVEN / RELABEL: the caller's arrays;
-  // else empty).  Labels start stale (psi = 0 < base).
-  __device__ void init_state() {
+  // Vertex state from the initial matching (GIVEN / RELABEL / UNIT: the caller's
+  // arrays; else empty).  Labels start stale (psi = 0 < base), except in MODE_UNIT.
+  // Returns this thread's count of out-of-range inputs.
+  __device__ long long init_state() {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     if (p.mode == MODE_GAP) {
       for (int u = g; u < m; u += G) {
@@ -447,17 +454,43 @@ struct Solver {
         int l = p.cmatch_in[v];
         vst(p.colst + v, pack(-1, (l >= 0 && l < INF) ? 1u + (u32)l : 0u));
       }
-      return;
+      return 0;
     }
-    const bool given = (p.mode == MODE_RELABEL) || (p.init == 1);
+    // a caller's matching (GIVEN solve, relabel, unit) is range-checked here: a bad
+    // entry is counted (-> MCM_EINVAL after the barrier) and read as -1, so no
+    // later phase can index outside rowst / colst.  Columns may carry the internal
+    // -2 ("dead") mark in the relabel and unit modes only.
+    const bool given = p.mode == MODE_RELABEL || p.mode == MODE_UNIT || (p.mode == MODE_SOLVE && p.init == 1);
+    const int cmin = p.mode == MODE_SOLVE ? -1 : -2;
+    const bool unit = p.mode == MODE_UNIT;
+    long long bad = 0, dead = 0;
     for (int u = g; u < m; u += G) {
-      vst(p.rowst + u, pack(given ? p.rmatch_in[u] : -1, 0));
+      int x = given ? p.rmatch_in[u] : -1;
+      if (x < -1 || x >= n) { bad++; x = -1; }
+      vst(p.rowst + u, pack(x, unit ? enc_label(p.psi_row_io[u]) : 0u));
     }
     for (int v = g; v < n; v += G) {
-      vst(p.colst + v, pack(given ? p.cmatch_in[v] : -1, 0));
-      p.iA[v] = -1;  // R12
+      int x = given ? p.cmatch_in[v] : -1;
+      if (x < cmin || x >= m) { bad++; x = -1; }
+      dead += x == -2;
+      vst(p.colst + v, pack(x, unit ? enc_label(p.psi_col_io[v]) : 0u));
+      if (!unit) p.iA[v] = -1;  // R12 (unit: the caller's iA)
     }
+    if (unit)
+      for (int i = g; i < p.unit_len; i += G) {
+        const int a = p.wl0[i], b = p.wl1[i];
+        bad += (a < -1 || a >= n) + (b < -1 || b >= n);
+        if (a < -1 || a >= n) p.wl0[i] = -1;
+        if (b < -1 || b >= n) p.wl1[i] = -1;
+      }
+    // relabel mode: -2 columns count as dead for the early-stop target (R22)
+    dead = cta_sum<NT>(dead, sm.red);
+    if (threadIdx.x == 0 && dead && p.mode == MODE_RELABEL) atomicAdd(&p.ctrl->ndead, (u32)dead);
+    return bad;
   }
+  // label l of a caller (MODE_UNIT) -> stored word value at base 1: 1 + l when
+  // finite, 0 (stale = m+n) otherwise
+  __device__ __forceinline__ u32 enc_label(int l) const { return (l >= 0 && l < INF) ? 1u + (u32)l : 0u; }
 
   // Cheap greedy matching on the device (reading R13): every column claims the
   // first free row of Gamma(v) with a CAS.  A column fails only when every
@@ -1757,6 +1790,23 @@ struct Solver {
     if (GRID && MCM_FINE) tmark(106, 0);
     if (lead()) L().ns_gr += (long long)(tnow() - g0);
   }
+  // SHRKRNL: the fix step of every slot (fix_slots, Alg. 8) with the
+  // surviving columns compacted to Ac[0 ..) in slot order (two passes over the CTAs'
+  // chunks; T = scratch of len entries); returns the new length.
+  template <bool GRID>
+  __device__ int fix_compact(int len, int *Ac, const int *Ap, int lp, int *T) {
+    if (lead()) S(SS_SLOTS) += len;
+    const int r1 = (GRID && len > 2 * NT * ncta<GRID>())
+                       ? compact_pass1<GRID, 4>(len, [&](int i0, int hi, int *val) { fix_slots<4>(i0, hi, Ac, Ap, lp, val); },
+                                                T, Ac)
+                       : compact_pass1<GRID, 1>(len, [&](int i0, int hi, int *val) { fix_slots<1>(i0, hi, Ac, Ap, lp, val); },
+                                                T, Ac);
+    barrier<GRID, false>();
+    if (ncta<GRID>() == 1) return r1;
+    len = compact_pass2<GRID>(len, T, Ac, r1);
+    barrier<GRID, false>();  // Ac was rewritten by other CTAs: order it before PUSH
+    return len;
+  }
   // one iteration of Alg. 7 l.10-19: fix step (INITKRNL, or SHRKRNL = fix + stable
   // compaction), then PUSHKRNL and the Ac/Ap swap.  Returns false when the fix
   // step found no active column.  The tail group compacts at every step.
@@ -1768,19 +1818,7 @@ struct Solver {
     int act;
     trace(3, c.len);
     if (!GRID || (c.shrink && p.shrink_min >= 0 && c.len >= p.shrink_min) || p.compact_every || c.compact_next) {
-      if (lead()) S(SS_SLOTS) += c.len;
-      int r1 = (GRID && c.len > 2 * NT * ncta<GRID>())
-                   ? compact_pass1<GRID, 4>(c.len, [&](int i0, int hi, int *val) { fix_slots<4>(i0, hi, Ac, Ap, lp, val); },
-                                            Tb(c), Ac)
-                   : compact_pass1<GRID, 1>(c.len, [&](int i0, int hi, int *val) { fix_slots<1>(i0, hi, Ac, Ap, lp, val); },
-                                            Tb(c), Ac);
-        barrier<GRID, false>();
-      if (ncta<GRID>() > 1) {
-        c.len = compact_pass2<GRID>(c.len, Tb(c), Ac, r1);
-        barrier<GRID, false>();  // Ac was rewritten by other CTAs: order it before PUSH
-      } else {
-        c.len = r1;
-      }
+      c.len = fix_compact<GRID>(c.len, Ac, Ap, lp, Tb(c));
       act = c.len;
       if (c.shrink && lead()) L().shrinks++;
       c.shrink = 0;
@@ -1872,8 +1910,10 @@ struct Solver {
         if (c.gr_active) {
           if (c.gst.nlen > up) { reason = R_GRID; break; }
           gr_step<false>(c);
+          if (lead()) L().tail_levels++;
           continue;
         }
+        if ((F & F_AUX) && p.mode == MODE_RELABEL && c.loop != c.iterGR) { reason = R_TERM; break; }  // GR done
         if (c.loop == c.gapAt) { reason = R_GRID; break; }
         if (c.loop == c.iterGR) {
           if (c.ulen > up || base_overflow(c)) { reason = R_GRID; break; }
@@ -2030,59 +2070,54 @@ struct Solver {
   // Stale rows (R27, build addition): at termination a row u with mu(u) = c whose
   // column does not point back (mu(c) != u).  The paper argues that only column
   // entries of mu can be inconsistent when the loop ends.  Push chains
-  // (R26) claim rows by CAS but store mu(c) plainly, and when c is displaced from
-  // a row and pushed on by another chain before the first chain's store of mu(c)
-  // has landed, that late store leaves mu(c) naming the row c was displaced from
-  // (seen under compute-sanitizer's slowed schedule; 0 in 600 plain solves).  A
-  // stale row would count in |M| and never start a BFS.  So before the guard's GR:
-  // if c's own row does not point back either, c is re-attached to u (CAS on
-  // c's word, so one row wins when several hold c); otherwise, or when the CAS
-  // loses, u is set unmatched and appended to U, and the guard's GR then reaches
-  // every unmatched column an augmenting path still leads to.  One pass over the
-  // row words (plus the mates' column words).
+  // (R26) claim rows by CAS and then set mu(c) by CAS (chain_settle); a late
+  // setting can still lose against a newer push of c, and a caller's GIVEN matching
+  // may hold such rows too.  A stale row would count in |M| and never start a BFS.
+  // So before the guard's GR: if c's own row does not point back either, c is
+  // re-attached to u (CAS on c's word, so one row wins when several hold c);
+  // otherwise, or when the CAS loses, u is set unmatched.  The same pass rebuilds
+  // the unmatched-row list U from scratch (every row unmatched after the repair,
+  // isolated rows excepted, each once), so the guard's GR starts from every
+  // unmatched row and U can never overflow.  One pass over the row words (plus the
+  // mates' column words and the bounds of the unmatched rows).
   __device__ void repair_rows(Ctl &c) {
     int *U = Ub(c);
-    const int cap = max(m, n) + 1;
-    long long fixedc = 0, freed = 0;
+    long long repaired = 0;
     for (int t = blockIdx.x * NT; t < m; t += gridDim.x * NT) {
       const int u = t + (int)threadIdx.x;
       u64 w = 0, cw = 0;
       int cc = -1;
-      bool stale = false;
+      bool stale = false, unm = false;
       if (u < m) {
         w = vld(p.rowst + u);
         cc = mu_of(w);
         if (cc >= 0) {
           cw = ld_rlx(p.colst + cc);
           stale = mu_of(cw) != u;
+        } else {
+          unm = true;
         }
       }
-      bool drop = false;
       if (stale) {
         const int u2 = mu_of(cw);
         const bool c_free = u2 < 0 || mu_of(ld_rlx(p.rowst + u2)) != cc;
         if (c_free && atomicCAS(p.colst + cc, cw, pack(u, psi_of(cw))) == cw) {
           if (u2 == -2) atomicSub(&p.ctrl->ndead, 1u);
-          fixedc++;
         } else {
           vst(p.rowst + u, pack(-1, psi_of(w)));
-          drop = true;
-          freed++;
+          unm = true;
         }
+        repaired++;
       }
-      if (drop) {
-        cg::coalesced_group g = cg::coalesced_threads();
-        u32 b = 0;
-        if (g.thread_rank() == 0) b = atomicAdd(ring_now(6), (u32)g.size());
-        b = g.shfl(b, 0);
-        const long long at = (long long)c.ulen + b + g.thread_rank();
-        if (at < cap) U[at] = u;
-      }
+      if (unm && ld_ro(p.rptr + u) == ld_ro(p.rptr + u + 1)) unm = false;  // isolated: never in U (n_iso)
+      int tot, r = cta_rank<NT>(unm, sm.w, &tot);
+      if (threadIdx.x == 0) sm.qbase = tot ? (int)atomicAdd(ring_now(6), (u32)tot) : 0;
+      __syncthreads();
+      if (unm) U[sm.qbase + r] = u;
     }
-    add_count(fixedc + freed, 7);
+    add_count(repaired, 7);
     barrier<true>();
-    const int nr = (int)ring_prev(6);
-    if (nr) c.ulen = (int)min((long long)c.ulen + nr, (long long)cap);
+    c.ulen = (int)ring_prev(6);
     if (lead()) L().repaired += ring_prev(7);
   }
 
@@ -2131,11 +2166,26 @@ struct Solver {
     if (threadIdx.x == 0) { sm.qcnt = 0; sm.nhuge = 0; sm.nd = 0; sm.chmax = 0; memset(&sm.ld, 0, sizeof(LeadStats)); }
     for (int k = 0; k < SS_N; k++) sm.ts[k][threadIdx.x] = 0;
     if (threadIdx.x < 2) sm.lvc[threadIdx.x] = 0;
-    init_state();
-    barrier<true, false>();
-    if (p.mode == MODE_SOLVE && p.init == 0) {
+    add_count(init_state(), 7);
+    barrier<true>();
+    if (ring_prev(7)) {  // a caller's array held an out-of-range entry
+      if (lead()) p.ctrl->err = -1;  // MCM_EINVAL
+      return;
+    }
+    if ((F & F_AUX) && p.mode == MODE_UNIT) {  // mcm_unit_step: one phase on the caller's state
+      unit();
+      finish_stats(0, 0, 0);
+      return;
+    }
+    if ((p.mode == MODE_SOLVE && p.init == 0) || p.mode == MODE_INIT) {
       greedy();
       barrier<true, false>();
+    }
+    if ((F & F_AUX) && p.mode == MODE_INIT) {  // mcm_initial_matching: M0 out, |M0| -> ring 0
+      fixmatching(0, 1);
+      barrier<true>();
+      finish_stats(0, 0, 0);
+      return;
     }
     debug_check(1, -1, nullptr, 0);
     // unmatched rows -> U; unmatched columns (increasing id) -> Ac (R12)
@@ -2143,7 +2193,8 @@ struct Solver {
     // isolated columns stay out of the worklist and count as dead (R25), except in
     // serial mode (the simulator's worklist holds every unmatched column, R12) and
     // in G-PR-First (no worklist: its loop tests and kills them itself)
-    const bool skip_iso = p.mode == MODE_SOLVE && !((F & F_SERIAL) && p.serial) && !((F & F_FIRST) && p.variant == 1);
+    const bool skip_iso = (p.mode == MODE_SOLVE || p.mode == MODE_RELABEL) && !((F & F_SERIAL) && p.serial) &&
+                          !((F & F_FIRST) && p.variant == 1);
     long long iso_c = 0;
     int run1 = compact_pass1<true, 8>(
         n, [&](int i0, int hi, int *val) { iso_c += cols_unmatched<8>(i0, hi, val, skip_iso); }, T, Ac);
@@ -2162,11 +2213,8 @@ struct Solver {
       finish_stats(0, 0, 0);
       return;
     }
-    if ((F & F_AUX) && p.mode == MODE_RELABEL) {
-      int g;
-      int ml = global_relabel<true>(U, ulen, T, Qa, Qb, 1, nullptr, g);
-      write_labels(1);
-      if (lead()) p.ctrl->stat[ST_MAXLEVEL] = ml;
+    if ((F & F_AUX) && p.mode == MODE_RELABEL) {  // mcm_global_relabel: one GR as a solve would run it
+      relabel(ulen);
       finish_stats(0, 0, 0);
       return;
     }
@@ -2233,6 +2281,100 @@ struct Solver {
     finish_stats(init_card, ns_init, (long long)(tnow() - tA));
   }
 
+  // mcm_global_relabel (MODE_RELABEL): one GR on the caller's matching, run by the
+  // same state machine as a solve's GR -- grid levels, single-CTA tail levels with
+  // the frontier in shared memory (tail_max > 0, frontiers of at most tail_f rows,
+  // hand-over both ways), bottom-up levels (bu_div), and the early stop of R22 /
+  // R28 when gr_early is set (unreached vertices then carry the lower bounds
+  // floor_r / floor_c instead of m+n).  Writes the decoded labels; stats slots:
+  // maxLevel (as GETITERGR sees it), the floors and the levels run in the tail.
+  __device__ void relabel(int ulen) {
+    Ctl c;
+    memset(&c, 0, sizeof(c));
+    c.ulen = ulen; c.base = 1; c.gapAt = -1; c.ac0 = 1; c.u0 = 1;  // loop = iterGR = 0: the GR is due
+    c.floor_r = c.floor_c = INF;
+    const int up = tail_f();
+    for (;;) {
+      if (!c.gr_active && c.loop != c.iterGR) break;  // gr_finish moved iterGR past loop: done
+      const bool tail_ok = p.tail_max > 0 && (c.gr_active ? c.gst.nlen <= up / 2 : c.ulen <= up);
+      if (tail_ok) tail_episode(c);
+      else if (c.gr_active) gr_step<true>(c);
+      else gr_begin<true>(c);
+    }
+    const u32 base = c.base - stride();  // gr_finish moved base to the next epoch
+    const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    for (int u = g; u < m; u += G) p.rmatch_out[u] = labf(psi_of(vld(p.rowst + u)), base, c.floor_r);
+    for (int v = g; v < n; v += G) p.cmatch_out[v] = labf(psi_of(vld(p.colst + v)), base, c.floor_c);
+    if (lead()) {
+      p.ctrl->stat[ST_MAXLEVEL] = c.gst.deepest + 2;
+      p.ctrl->stat[ST_FLOOR_R] = c.floor_r;
+      p.ctrl->stat[ST_FLOOR_C] = c.floor_c;
+    }
+    barrier<true, false>();
+  }
+
+  // mcm_unit_step (MODE_UNIT): ONE phase of the solve on the caller's state (mu,
+  // labels at base 1, iA, Ac = wl0, Ap = wl1, loop), run by the code a solve runs:
+  // on the grid (every CTA) or in the single-CTA tail (CTA 0, the worklist in
+  // shared memory when it fits, as tail_episode keeps it).  Result -> stat slot
+  // ST_MAXLEVEL: FIX the active-slot count, SHRINK the new length, FIXMATCHING |M|.
+  __device__ void unit() {
+    const u32 base = 1;
+    fl_r = fl_c = INF;
+    const int lp = (int)p.unit_loop, len = p.unit_len, what = p.unit_what;
+    int *Ac = p.wl0, *Ap = p.wl1;
+    long long r = 0;
+    if (p.unit_where == 0 || what == UNIT_FIXMATCHING) {
+      if (what == UNIT_FIX) {
+        fix_plain<true>(len, Ac, Ap, lp, 0);
+        barrier<true>();
+        r = ring_prev(0);
+      } else if (what == UNIT_SHRINK) {
+        r = fix_compact<true>(len, Ac, Ap, lp, p.qb);
+      } else if (what == UNIT_PUSH) {
+        push<true>(len, Ac, Ap, lp, base);
+        barrier<true, false>();
+      } else {
+        fixmatching(0, 1);
+        barrier<true>();
+        r = ring_prev(0);
+      }
+    } else {
+      if (blockIdx.x == 0) {
+        const bool sh = len <= TW;  // tail_episode's wl_in
+        for (int i = threadIdx.x; sh && i < len; i += NT) { sm.wl[0][i] = __ldcg(Ac + i); sm.wl[1][i] = __ldcg(Ap + i); }
+        __syncthreads();
+        int *A = sh ? sm.wl[0] : Ac, *B = sh ? sm.wl[1] : Ap;
+        if (what == UNIT_PUSH) push<false>(len, A, B, lp, base);
+        else r = fix_compact<false>(len, A, B, lp, nullptr);  // the tail compacts at every fix step
+        __syncthreads();
+        for (int i = threadIdx.x; sh && i < len; i += NT) { Ac[i] = sm.wl[0][i]; Ap[i] = sm.wl[1][i]; }
+        if (threadIdx.x == 0) {
+          p.ctrl->ho_ph = ph;
+          p.ctrl->ho[0] = r;
+          for (int j = 0; j < 4; j++)
+            for (int q = 0; q < 8; q++) p.ctrl->ring[j][q] = 0;
+        }
+      }
+      grid_sync(&p.ctrl->bar, true, [&] { load_handover(); });
+      ph = sm.ho_ph + 1;
+      r = sm.ho[0];
+    }
+    const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    for (int u = g; u < m; u += G) {
+      const u64 w = vld(p.rowst + u);
+      if (what != UNIT_FIXMATCHING) p.rmatch_out[u] = mu_of(w);
+      p.psi_row_io[u] = labf(psi_of(w), base, INF);
+    }
+    for (int v = g; v < n; v += G) {
+      const u64 w = vld(p.colst + v);
+      if (what != UNIT_FIXMATCHING) p.cmatch_out[v] = mu_of(w);
+      p.psi_col_io[v] = labf(psi_of(w), base, INF);
+    }
+    if (lead()) p.ctrl->stat[ST_MAXLEVEL] = r;
+    barrier<true, false>();
+  }
+
   __device__ void reset_labels() {
     const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
     for (int u = g; u < m; u += G) {
@@ -2260,8 +2402,9 @@ struct Solver {
       st[ST_NS_LOOP] = l.ns_loop; st[ST_NS_TOTAL] = ns_total; st[ST_TAILLOOPS] = l.tail_loops;
       st[ST_BARRIERS] = l.nbar;
       st[ST_REPAIRED] = l.repaired;
+      st[ST_TAIL_LEVELS] = l.tail_levels;
       st[ST_TRACE_N] = l.tn;
-      if (p.mode == MODE_SOLVE) {
+      if (p.mode == MODE_SOLVE || p.mode == MODE_INIT) {
         st[ST_CARD] = (long long)ring_prev(0);
         st[ST_FIXED] = (long long)ring_prev(1);
       }

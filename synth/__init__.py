@@ -274,3 +274,65 @@ def random_small(m: int, n: int, p: float, seed: int) -> Graph:
     mask = rng.random((m, n)) < p
     r, c = np.nonzero(mask)
     return from_pairs(m, n, r, c, f"er{m}x{n}")
+
+
+# ---------------------------------------------------------------- unit-step inputs
+def push_instance(K: int, seed: int, loop: int = 5, deg_mix=((0.6, 1, 8), (0.25, 9, 64), (0.1, 65, 512),
+                                                             (0.05, 513, 3000)),
+                  p_mate=0.5, p_inf=0.1, p_dead=0.05, p_empty=0.05, p_inf_col=0.02, p_blocked=0.3):
+    """A PUSHKRNL input (Alg. 9) whose active columns do not interact, so a parallel
+    push is deterministic: K active columns, each with a PRIVATE set of rows (no row
+    is adjacent to two active columns); a row may be matched to a private "mate"
+    column w (G(w) = {that row}, w not in the worklist).  Labels respect the
+    neighbourhood invariant psi(u) >= psi(v) - 1 on every edge of an active column
+    (P:203-209), under which the first minimum of a chunked scan equals the serial
+    one (reading R11).  Degrees follow deg_mix (fraction, min, max) so lane groups,
+    warps and CTA-wide scans all occur.  Pure input construction: no matching
+    arithmetic.  Returns (graph, state) with state = dict(mu_row, mu_col, psi_row,
+    psi_col, iA, Ac, loop) as int32 arrays (INF = m + n)."""
+    rng = np.random.default_rng(seed)
+    fr = np.array([f for f, _, _ in deg_mix])
+    kind = rng.choice(len(deg_mix), size=K, p=fr / fr.sum())
+    lo = np.array([a for _, a, _ in deg_mix])[kind]
+    hi = np.array([b for _, _, b in deg_mix])[kind]
+    deg = rng.integers(lo, hi + 1)
+    R = int(deg.sum())
+    owner = np.repeat(np.arange(K), deg)              # active column (local id) of each private row
+    has_mate = rng.random(R) < p_mate
+    nm = int(has_mate.sum())
+    m, n = R, K + nm
+    INF = m + n
+    rperm = rng.permutation(m)                        # row ids shuffled
+    cperm = rng.permutation(n)                        # column ids shuffled (active: local 0..K-1, mates: K..)
+    row_id = rperm[np.arange(R)]
+    act_id = cperm[np.arange(K)]
+    mate_id = np.full(R, -1, np.int64)
+    mate_id[has_mate] = cperm[K + np.arange(nm)]
+    rows = np.concatenate([row_id, row_id[has_mate]])
+    cols = np.concatenate([act_id[owner], mate_id[has_mate]])
+    g = from_pairs(m, n, rows, cols, name=f"push_instance(K={K},seed={seed})")
+    mu_row = np.full(m, -1, np.int32)
+    mu_col = np.full(n, -1, np.int32)
+    mu_row[row_id[has_mate]] = mate_id[has_mate]
+    mu_col[mate_id[has_mate]] = row_id[has_mate]
+    psi_row = np.full(m, INF, np.int32)
+    psi_col = rng.integers(1, 2 * INF if INF < 40 else 40, n).astype(np.int32)
+    psi_col = np.minimum(psi_col, INF)
+    pv = rng.integers(1, 30, K)
+    pv[rng.random(K) < p_inf_col] = INF               # label already infinite (R19 when dead_skip)
+    psi_col[act_id] = pv
+    base = np.maximum(pv[owner] - 1, 0)
+    lab = base + rng.integers(0, 12, R)
+    lab[rng.random(R) < p_inf] = INF
+    lab[np.isin(owner, np.nonzero(rng.random(K) < p_dead)[0])] = INF   # every row infinite: the column dies
+    psi_row[row_id] = np.minimum(lab, INF)
+    iA = rng.integers(-1, loop, n).astype(np.int32)
+    blk = has_mate & (rng.random(R) < p_blocked)
+    iA[mate_id[blk]] = loop                           # the displaced column was active this loop: blocked
+    iA[act_id] = loop                                 # the fix step marked the active columns
+    Ac = act_id[rng.permutation(K)].astype(np.int64)
+    empty = rng.random(K) < p_empty
+    Ac[empty] = -1
+    state = dict(mu_row=mu_row, mu_col=mu_col, psi_row=psi_row, psi_col=psi_col.astype(np.int32), iA=iA,
+                 Ac=Ac.astype(np.int32), loop=loop)
+    return g, state
