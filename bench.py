@@ -52,6 +52,13 @@ METRIC = "MCM solve throughput (edges/s = nnz / (create + solve time)) per graph
 PAPER_OPTS = dict(tail_chain=0, grid_chain=0, gr_early=0, compact_adapt=0, k=0.7)
 
 
+def config_keys(name, g, l2, parallelism):
+    """The `config` object: the same keys on both arms (workload, sizes, L2 policy,
+    parallelism); run details go to `run`."""
+    return {"workload": f"{name}: {CONFIG_DESC[name]}", "m": g.m, "n": g.n, "nnz": g.nnz, "l2": l2,
+            "parallelism": parallelism}
+
+
 def _peaks():
     try:
         return json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))
@@ -319,15 +326,14 @@ def run_ours(args, rank, world, local_rank):
         "vs_baseline": None,
         "dtype": "int32",
         "data": "synthetic",
-        "config": {
-            "workload": f"{args.config}: {CONFIG_DESC[args.config]}",
-            "m": g.m, "n": g.n, "nnz": g.nnz, "mm": cards[-1], "init_card": stats["init_card"],
+        "config": config_keys(args.config, g, "flushed between steps (512 MiB write, outside the step events)",
+                              f"replicas x{world} (one instance per GPU, no collective)"),
+        "run": {
+            "mm": cards[-1], "init_card": stats["init_card"],
             "options": used_opts,
             "step": "mcm_create + mcm_solve (device-resident CSR)",
             "ms_create": t_create_max, "ms_solve": t_solve_max,
             "edges_per_s_solve_only": nnz_total / (t_solve_max * 1e-3),
-            "l2": "flushed between steps (512 MiB write, outside the step events)",
-            "parallelism": f"replicas x{world} (one instance per GPU, no collective)",
             "wall_s_timed_region": wall,
         },
         "roofline": {
@@ -362,7 +368,7 @@ def run_ours(args, rank, world, local_rank):
         "paper_config": paper_config,
     }
     if world > 1:
-        line["config"]["nccl_world_size"] = world
+        line["run"]["nccl_world_size"] = world
     if world == 1 and not args.no_cpu_baseline:
         line["cpu_baseline"] = cpu_baseline(args.config, g)
     return line
@@ -466,6 +472,17 @@ def mt_init(mt, ip, ix, g, ws, opts, stream=None):
     mt._h = h
 
 
+def batch_partition(batch, world, rank):
+    """C5: graph i of the batch goes to rank i mod world; no collective."""
+    return [i for i in range(batch) if i % world == rank]
+
+
+def batch_graphs(indices, scale=1.0):
+    import synth
+
+    return [synth.config("C5", scale, index=i) for i in indices]
+
+
 def run_batch(args, rank, world, local_rank):
     """C5 (BASELINE configs[4]): a batch of args.batch independent 2^21 x 2^21 graphs;
     rank r solves graphs r, r+N, ... (no collective).  On one GPU the rank's graphs
@@ -481,11 +498,11 @@ def run_batch(args, rank, world, local_rank):
 
     dev = torch.device("cuda", local_rank)
     torch.cuda.set_device(dev)
-    mine = [i for i in range(args.batch) if i % world == rank]
+    mine = batch_partition(args.batch, world, rank)
     S = max(1, min(args.streams, len(mine)))
     sms = torch.cuda.get_device_properties(dev).multi_processor_count
     opts = dict(k=args.k, grid_ctas=max(1, sms // S))
-    graphs = [synth.config("C5", 1.0, index=i) for i in mine]
+    graphs = batch_graphs(mine)
     host = [(torch.from_numpy(g.indptr).pin_memory(), torch.from_numpy(g.indices).pin_memory()) for g in graphs]
     devg = [(a.to(dev), b.to(dev)) for a, b in host]
     streams = [torch.cuda.Stream(dev) for _ in range(S)]
@@ -585,12 +602,13 @@ def run_batch(args, rank, world, local_rank):
         "metric": METRIC, "value": nnz_total / (t_step_max * 1e-3), "unit": "edges/s", "n_gpus": world,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": t_step_max, "higher_is_better": True,
         "scaling": "strong", "vs_baseline": None, "dtype": "int32", "data": "synthetic",
-        "config": {"workload": f"C5: batch of {args.batch} x ({CONFIG_DESC['C5']})", "graphs_per_rank": len(graphs),
-                   "streams_per_gpu": S, "ctas_per_solve": opts["grid_ctas"], "nnz_rank0": int(nnz_rank),
-                   "cards_rank0": sorted(set(cards)), "k": args.k,
-                   "step": "every graph of the rank: mcm_create + mcm_solve (device-resident CSRs), S concurrent streams",
+        "config": {"workload": f"C5: batch of {args.batch} x ({CONFIG_DESC['C5']})", "m": graphs[0].m,
+                   "n": graphs[0].n, "nnz": int(nnz_total),
                    "l2": "flushed between steps (512 MiB write, outside the step events)",
                    "parallelism": f"batch over {world} GPU(s), graph i on rank i mod {world}, no collective"},
+        "run": {"graphs_per_rank": len(graphs), "streams_per_gpu": S, "ctas_per_solve": opts["grid_ctas"],
+                "nnz_rank0": int(nnz_rank), "cards_rank0": sorted(set(cards)), "k": args.k,
+                "step": "every graph of the rank: mcm_create + mcm_solve (device-resident CSRs), S concurrent streams"},
         "roofline": {"bound": "hbm", "kernel": "gpr_kernel (all concurrent solves of a step)", "achieved": achieved,
                      "peak": hbm_peak, "unit": "GB/s", "frac": achieved / hbm_peak, "traffic": None,
                      "algorithmic_bytes_per_launch": alg // len(graphs),
@@ -603,6 +621,7 @@ def run_batch(args, rank, world, local_rank):
                 "h2d_bytes_per_step": int(sum(4 * (g.m + 1 + g.nnz) for g in graphs)),
                 "d2h_bytes_per_step": int(sum(4 * (g.m + g.n) for g in graphs)), "ms_per_step": t_e2e_max},
         "gpu_launches": args.steps * sum(st_["kernel_launches"] for st_ in stats),
+        "nccl_world_size": world,
     }
     if world == 1 and not args.no_cpu_baseline:
         line["cpu_baseline"] = cpu_baseline("C5", graphs[0])
@@ -704,7 +723,7 @@ def run_reference(args, rank):
         "impl": "reference", "metric": METRIC, "value": v, "unit": "edges/s", "n_gpus": 1, "steps": args.steps,
         "warmup": args.warmup, "ms_per_step": t * 1e3, "higher_is_better": True, "scaling": "weak",
         "vs_baseline": None, "dtype": "int32", "data": "synthetic",
-        "config": {"workload": f"{args.config}: {CONFIG_DESC[args.config]}", "m": g.m, "n": g.n, "nnz": g.nnz},
+        "config": config_keys(args.config, g, "n/a (host run)", "host, 1 core (oracle)"),
         "cpu_baseline": {"value": v, "unit": "edges/s", "cores": 1, "kind": "oracle",
                          "sample": f"full {args.config} graph per step: cheap matching + sequential PR-FIFO "
                                    f"(k=0.5), single core", **info},
@@ -738,6 +757,9 @@ def main():
 
         torch.cuda.set_device(local_rank)
         torch.distributed.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
+        if rank == 0:  # the driver's scaling run can check that NCCL saw every rank
+            print(f"[bench] torch.distributed backend {torch.distributed.get_backend()}, world size "
+                  f"{torch.distributed.get_world_size()}", file=sys.stderr, flush=True)
     line = (run_batch if args.config == "C5" else run_ours)(args, rank, world, local_rank)
     if line:
         print(json.dumps(line), flush=True)

@@ -11,7 +11,7 @@ import oracle  # noqa: E402
 import synth  # noqa: E402
 
 CASES = [("C1", 1.0), ("C1", 0.1), ("C2", 0.01), ("C2", 0.1), ("C3", 0.001), ("C3", 0.01), ("C4", 1 / 1024),
-         ("C4", 1 / 64), ("C5", 1 / 256), ("C5", 1 / 16)]
+         ("C4", 1 / 64), ("C5", 1 / 256), ("C5", 1 / 16), ("C2", 1.0), ("C3", 1.0), ("C4", 1.0), ("C5", 1.0)]
 
 
 def main():
