@@ -140,6 +140,13 @@ typedef struct {
   int32_t gr_target_min; /* gr_target applies only to GRs that start with at least this many
                            alive unmatched columns (fewer: every one must be labelled);
                            default 1024 */
+  int32_t gr_concurrent; /* concurrent GR and push (the paper's future work; SURVEY
+                           NEXT-2; an experiment): > 0 = a second persistent kernel on
+                           this many CTAs runs complete GRs into shadow labels, on a stream of
+                           the handle's own, while the solve kernel (the remaining CTAs) keeps
+                           pushing; finished labels are installed at the next loop boundary.
+                           The exactness guard keeps the result exact.  Ignored in serial mode
+                           and for G-PR-First.  Default 0 (off). */
 } mcm_options_t;
 
 typedef struct {

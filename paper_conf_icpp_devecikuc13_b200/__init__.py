@@ -63,6 +63,7 @@ class Options(ctypes.Structure):
         ("max_loops", ctypes.c_int64),
         ("gr_target", ctypes.c_double),
         ("gr_target_min", ctypes.c_int32),
+        ("gr_concurrent", ctypes.c_int32),
     ]
 
 

@@ -24,7 +24,8 @@ constexpr int MAX_CTAS = 4096;
 size_t align256(size_t x) { return (x + 255) & ~(size_t)255; }
 
 struct Layout {
-  size_t ctrl, ovf, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, outr, outc, dbg, total;
+  size_t ctrl, ovf, rptr, radj, cptr, cadj, rowst, colst, iA, wl0, wl1, q[4], ctacnt, bsum, hist, outr, outc, dbg, ctrl2,
+      srow, scol, total;
   int hist_len;
 };
 
@@ -55,6 +56,10 @@ Layout layout(int32_t m, int32_t n, int64_t nnz) {
   L.outr = take(sizeof(int) * (size_t)m);  // mcm_match_host: device copy of the matching
   L.outc = take(sizeof(int) * (size_t)n);
   L.dbg = take(sizeof(int) * ((size_t)n + 1) + (getenv("MCM_TRACE") ? (size_t)atoi(getenv("MCM_TRACE")) * 24 : 0));
+  // concurrent GR (option gr_concurrent): the GR kernel's control block and shadow labels
+  L.ctrl2 = take(sizeof(Ctrl));
+  L.srow = take(sizeof(u32) * (size_t)m);
+  L.scol = take(sizeof(u32) * (size_t)n);
   L.total = o;
   return L;
 }
@@ -202,6 +207,13 @@ struct mcm_ctx {
   mcm_stats_t stats;
   double ms_setup = 0;
   int create_launches = 0;
+  cudaStream_t s2 = nullptr;  // concurrent GR: the GR kernel's stream (created on first use)
+  cudaEvent_t e1 = nullptr, e2 = nullptr;
+  ~mcm_ctx() {
+    if (s2) cudaStreamDestroy(s2);
+    if (e1) cudaEventDestroy(e1);
+    if (e2) cudaEventDestroy(e2);
+  }
   Ctrl host_ctrl;
 };
 
@@ -276,6 +288,7 @@ static int check_opts(const mcm_options_t *o) {
     return MCM_EINVAL;
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
   if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0 || o->grid_chain < 0) return MCM_EINVAL;
+  if (o->gr_concurrent < 0 || o->gr_concurrent > MAX_CTAS) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -330,14 +343,15 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
 
   int *cptr = (int *)(ws + L.cptr), *cadj = (int *)(ws + L.cadj);
   // CSC by counting sort (Gamma(v) for the push, Alg. 9 l.6): degrees
-  // (k_ingest), exclusive scan, scatter.  (A pass-blocked scatter that keeps each
-  // pass's cadj segment in L2 halved the DRAM writes on C4 but re-read radj once
-  // per pass: 5.3 ms against 3.0 ms, rejected.)
-  int nb = (n + SCAN_B - 1) / SCAN_B;
-  if (nb == 0) nb = 1;
-  k_scan_sums<<<nb, 512, 0, st>>>(cnt, n, bsum);
-  k_scan_bsum<<<1, 1024, 0, st>>>(bsum, nb);
-  k_scan_apply<<<nb, 1024, 0, st>>>(cnt, n, bsum, cptr, n);
+  // (k_ingest), exclusive scan, scatter.  (Rejected alternatives, measured: a
+  // pass-blocked scatter keeping each pass's cadj segment in L2, 5.3 ms on C4, round
+  // 1; a bucketed two-pass transpose, 6.2-8.7 ms on C4 and a slower C3 trajectory,
+  // round 2 -- DESIGN.md §7.)
+  int nsb = (n + SCAN_B - 1) / SCAN_B;
+  if (nsb == 0) nsb = 1;
+  k_scan_sums<<<nsb, 512, 0, st>>>(cnt, n, bsum);
+  k_scan_bsum<<<1, 1024, 0, st>>>(bsum, nsb);
+  k_scan_apply<<<nsb, 1024, 0, st>>>(cnt, n, bsum, cptr, n);
   nlaunch += 3;
   CK(cudaGetLastError());
   if (n == 0) CK(cudaMemsetAsync(cptr, 0, sizeof(int), st));
@@ -458,7 +472,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   int C = mode == MODE_UNIT ? 1 : o.tail_ctas;  // a unit's tail is CTA 0 alone
   // the lean production instance unless a feature only the full one carries is on
   // (a cluster tail group spans several SMs' L1s: it needs gpu-scope vertex state)
-  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1)
+  const bool conc = mode == MODE_SOLVE && o.gr_concurrent > 0 && !o.serial && !o.variant;
+  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1 || conc)
                                    ? gpr_kernel<F_ALL>
                                    : gpr_kernel<F_FAST>;
   if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
@@ -483,6 +498,37 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.tail_ctas = C;
   h->grid = grid;
   CK(cudaMemsetAsync(p.ctrl, 0, sizeof(Ctrl), st));
+  if (conc) {
+    // NEXT-2: the GR kernel on its own stream (ordered after everything enqueued on
+    // `st` so far), co-resident with the solve kernel, which keeps the other CTAs
+    const int A = std::min(o.gr_concurrent, grid - C);
+    if (A < 1) return MCM_EINVAL;
+    if (!h->s2) CK(cudaStreamCreateWithFlags(&h->s2, cudaStreamNonBlocking));
+    if (!h->e1) CK(cudaEventCreateWithFlags(&h->e1, cudaEventDisableTiming));
+    if (!h->e2) CK(cudaEventCreateWithFlags(&h->e2, cudaEventDisableTiming));
+    Ctrl *c2 = (Ctrl *)(ws + L.ctrl2);
+    p.ctrl2 = c2;
+    p.srow = (u32 *)(ws + L.srow);
+    p.scol = (u32 *)(ws + L.scol);
+    CK(cudaMemsetAsync(c2, 0, sizeof(Ctrl), st));
+    CK(cudaMemsetAsync(p.srow, 0, sizeof(u32) * (size_t)h->m, st));
+    CK(cudaMemsetAsync(p.scol, 0, sizeof(u32) * (size_t)h->n, st));
+    CK(cudaEventRecord(h->e1, st));
+    CK(cudaStreamWaitEvent(h->s2, h->e1, 0));
+    Params pg = p;
+    pg.mode = MODE_CONC_GR;
+    pg.ctrl = c2;
+    cudaLaunchConfig_t cg2 = {};
+    cudaLaunchAttribute a2[1];
+    a2[0].id = cudaLaunchAttributeCooperative;
+    a2[0].val.cooperative = 1;
+    cg2.gridDim = dim3(A); cg2.blockDim = dim3(NT); cg2.dynamicSmemBytes = sizeof(Smem); cg2.stream = h->s2;
+    cg2.attrs = a2; cg2.numAttrs = 1;
+    CK(cudaLaunchKernelEx(&cg2, gpr_kernel<F_ALL>, pg));
+    grid -= A;
+    p.conc = A;
+    h->grid = grid;
+  }
   cudaLaunchConfig_t cfg = {};
   cudaLaunchAttribute at[2];
   at[0].id = cudaLaunchAttributeCooperative;
@@ -492,6 +538,10 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   cfg.gridDim = dim3(grid); cfg.blockDim = dim3(NT); cfg.dynamicSmemBytes = sizeof(Smem); cfg.stream = st;
   cfg.attrs = at; cfg.numAttrs = C > 1 ? 2 : 1;
   CK(cudaLaunchKernelEx(&cfg, kern, p));
+  if (conc) {  // the solve's results are read after both kernels ended
+    CK(cudaEventRecord(h->e2, h->s2));
+    CK(cudaStreamWaitEvent(st, h->e2, 0));
+  }
   if (ua) {
     if (h->n) CK(cudaMemcpyAsync(ua->iA, p.iA, sizeof(int) * (size_t)h->n, cudaMemcpyDeviceToDevice, st));
     if (ua->len) {

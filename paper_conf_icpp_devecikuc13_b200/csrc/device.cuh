@@ -43,6 +43,10 @@ __device__ __forceinline__ void st_rlx(int *p, int v) {
 }
 // read-only graph arrays (never written during a solve)
 __device__ __forceinline__ int ld_ro(const int *p) { return __ldg(p); }
+// adjacency lists (radj / cadj): streamed, read-only.  (L2 evict_first hints on
+// these, and evict_last on the vertex state, were measured in round 2: within
+// noise on C2-C5, profiles/r02_l2hint_ab.txt; not kept.)
+__device__ __forceinline__ int ld_adj(const int *p) { return __ldg(p); }
 // phase-to-phase mutable arrays (worklists, queues): bypass L1
 __device__ __forceinline__ int ld_cg(const int *p) { return __ldcg(p); }
 __device__ __forceinline__ u32 ld_rlx(const u32 *p) {

@@ -23,6 +23,23 @@ namespace cg = cooperative_groups;
 #ifndef MCM_FINE
 #define MCM_FINE 0
 #endif
+// batch widths of the wide phases (independent items in flight per thread; capped
+// by the register budget: 512 threads x 128 registers)
+#ifndef MCM_RG
+#define MCM_RG 4   // greedy: columns per lane
+#endif
+#ifndef MCM_EB
+#define MCM_EB 4   // wide BFS level: adjacency entries per batch (two frontier entries per thread)
+#endif
+#ifndef MCM_PB
+#define MCM_PB 2   // wide push: slots per thread
+#endif
+#ifndef MCM_BUFLUSH
+#define MCM_BUFLUSH 16  // bottom-up BFS level: flush the staged frontier every this many tiles
+#endif
+#ifndef MCM_WFLUSH
+#define MCM_WFLUSH 0  // wide BFS level: flush the staged frontier every this many tiles (0: once per level)
+#endif
 namespace mcm {
 
 constexpr int NT = 512;          // threads per CTA
@@ -40,7 +57,7 @@ constexpr int HUGE_WARP = 8192;  // ... unless longer than this
 constexpr int KB = 4;            // neighbours in flight per lane (batched loads)
 constexpr int SPLIT = 1024;      // GR: a frontier row's adjacency is split into ranges of at most this many
 
-enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2, MODE_UNIT = 3, MODE_INIT = 4 };
+enum { MODE_SOLVE = 0, MODE_RELABEL = 1, MODE_GAP = 2, MODE_UNIT = 3, MODE_INIT = 4, MODE_CONC_GR = 5 };
 // mcm_unit_step: one phase of the solve on a given state (include/mcm.h)
 enum { UNIT_FIX = 0, UNIT_SHRINK = 1, UNIT_PUSH = 2, UNIT_FIXMATCHING = 3 };
 
@@ -66,6 +83,11 @@ struct Ctrl {
   // tail-mode handoff (tail group -> grid): reason, phase counter, Ctl image
   int ho_reason, ho_ph;
   long long ho[32];
+  // concurrent GR (option gr_concurrent): handshake between the push
+  // kernel and the GR kernel (fields of the GR kernel's own Ctrl block): requests
+  // (push -> GR), completions and the epoch of the finished labels (GR -> push),
+  // exit / exited, and the GR kernel's per-level frontier counters
+  u32 creq, cdone, cexit, cexited, csbase, ccnt[4];
 };
 
 struct Params {
@@ -106,6 +128,11 @@ struct Params {
   int *psi_row_io, *psi_col_io;
   int unit_what, unit_where, unit_len;
   long long unit_loop;
+  // concurrent GR (NEXT-2): CTAs of the GR kernel (0: off), its shadow labels, its
+  // control block
+  int conc;
+  u32 *srow, *scol;
+  Ctrl *ctrl2;
 };
 
 // per-CTA statistics accumulators (Smem::st), flushed at every barrier from
@@ -334,15 +361,12 @@ struct Solver {
     for (int c = s; c < e; c += SPLIT) stage(make_int4(w, c, min(e, c + SPLIT), c > s), next, gcnt);
   }
   // one more alive unmatched column labelled by this GR (ring counter 2): warp-
-  // aggregated into a per-CTA shared counter that flush() publishes once per tile
+  // aggregated into a per-CTA shared counter that flush() publishes once per level
   // (one global atomic per reached column put ~10^6 same-address atomics on one
   // L2 line in the first GRs of C3 / C4)
   __device__ __forceinline__ void count_free() {
     cg::coalesced_group g = cg::coalesced_threads();
-    if (g.thread_rank() == 0) {
-      if (sq) atomicAdd(ring_now(2), (u32)g.size());
-      else atomicAdd(&sm.lvc[0], (u32)g.size());
-    }
+    if (g.thread_rank() == 0) atomicAdd(&sm.lvc[0], (u32)g.size());
   }
   __device__ __forceinline__ void flush(int4 *next, u32 *gcnt) {
     if (sq) return;  // tail: the next frontier is the shared buffer itself
@@ -502,7 +526,7 @@ struct Solver {
     // the RG claims issued together, so a thread keeps RG independent chains in
     // flight; a column whose first free candidate was taken meanwhile (or that has
     // none among its first KB) continues alone from there.
-    constexpr int RG = 4;
+    constexpr int RG = MCM_RG;
     const int lane = lane_id();
     const int gw = (blockIdx.x * NT + threadIdx.x) >> 5, NWG = gridDim.x * NWARP;
     for (long long b = (long long)gw * 32 * RG; b < n; b += (long long)NWG * 32 * RG) {
@@ -523,7 +547,7 @@ struct Solver {
       for (int k = 0; k < RG; k++)
 #pragma unroll
         for (int q = 0; q < KB; q++)
-          u[k][q] = s[k] + q < e[k] ? ld_ro(p.cadj + s[k] + q) : -1;
+          u[k][q] = s[k] + q < e[k] ? ld_adj(p.cadj + s[k] + q) : -1;
 #pragma unroll
       for (int k = 0; k < RG; k++)
 #pragma unroll
@@ -563,7 +587,7 @@ struct Solver {
             int uu[KB];
             u64 rr[KB];
 #pragma unroll
-            for (int q = 0; q < KB; q++) uu[q] = j0 + q < e[k] ? ld_ro(p.cadj + j0 + q) : -1;
+            for (int q = 0; q < KB; q++) uu[q] = j0 + q < e[k] ? ld_adj(p.cadj + j0 + q) : -1;
 #pragma unroll
             for (int q = 0; q < KB; q++) rr[q] = uu[q] >= 0 ? vld(p.rowst + uu[q]) : 0ull;
 #pragma unroll
@@ -589,7 +613,7 @@ struct Solver {
             int j = c0 + lane;
             int uu = -1;
             u64 rr = 0;
-            if (j < eb) { uu = ld_ro(p.cadj + j); rr = vld(p.rowst + uu); S(SS_GYEDGES)++; }
+            if (j < eb) { uu = ld_adj(p.cadj + j); rr = vld(p.rowst + uu); S(SS_GYEDGES)++; }
             unsigned cand = __ballot_sync(0xffffffffu, uu >= 0 && mu_of(rr) == -1);
             while (cand && !dn) {
               int l = __ffs(cand) - 1;
@@ -686,6 +710,7 @@ struct Solver {
       // wide level: two frontier entries per thread per tile, their adjacency
       // expanded as one list in batches of 2*KB (twice the loads in flight of a
       // one-entry tile; the kernel's register budget caps the batch)
+      int wt = 0;
       for (int t = cta<GRID>() * 2 * NT; t < curlen; t += ncta<GRID>() * 2 * NT) {
         const int i0 = t + (int)threadIdx.x, i1 = i0 + NT;
         int4 q0 = i0 < curlen ? ld_q(cur4 + i0) : make_int4(-1, 0, 0, 0);
@@ -706,8 +731,12 @@ struct Solver {
             expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt, false);
           }
         }
-        flush(next, ncnt);
+        // every MCM_WFLUSH tiles (0: once per level): a flush is a few CTA barriers,
+        // and without it a wide level's output overflows the shared staging into the
+        // CTA's global overflow region (one more copy)
+        if (MCM_WFLUSH > 0 && ++wt % (MCM_WFLUSH > 0 ? MCM_WFLUSH : 1) == 0) flush(next, ncnt);
       }
+      flush(next, ncnt);
       return;
     }
     const int G = pick_group(curlen, ncta<GRID>() * NT);
@@ -727,10 +756,13 @@ struct Solver {
             u = -1;
           }
         }
-        int tot, r = cta_rank<NT>(keep, sm.w, &tot);
-        if (threadIdx.x == 0) sm.tmp = tot ? (int)atomicAdd(ucnt, (u32)tot) : 0;
-        __syncthreads();
-        if (keep) Uout[sm.tmp + r] = u;
+        if (keep) {  // filtered U: any order, one atomic per coalesced group (no CTA barrier;
+                     // a per-tile CTA reservation measured 10% slower on C4, equal on C3 / C5)
+          cg::coalesced_group kg = cg::coalesced_threads();
+          u32 b = 0;
+          if (kg.thread_rank() == 0) b = atomicAdd(ucnt, (u32)kg.size());
+          Uout[kg.shfl(b, 0) + kg.thread_rank()] = u;
+        }
         if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
       } else if (i < curlen) {
         int4 q = ld_q(cur4 + i);
@@ -748,9 +780,8 @@ struct Solver {
         expand(sb + lane, eb, 32, lc, lr, next, ncnt, guard, gcnt, false);
       }
       if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(103, 0);
-      flush(next, ncnt);
-      if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(104, 0);
     }
+    flush(next, ncnt);  // once per level
   }
   // Visit radj[j], j = j0, j0+step, ... < e, KB at a time.  A CAS claims each
   // column once per GR (so every row joins the next frontier once and every
@@ -766,7 +797,7 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         int jj = j + k * step;
-        v[k] = jj < e ? ld_ro(p.radj + jj) : -1;
+        v[k] = jj < e ? ld_adj(p.radj + jj) : -1;
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : ~0ull;
@@ -818,7 +849,7 @@ struct Solver {
   // load their mate)
   __device__ __forceinline__ void expand_pair(int d0, int s0, int d1, int s1, u32 lc, u32 lr, int4 *next, u32 *ncnt,
                                               int *guard, u32 *gcnt) {
-    constexpr int B = 2 * KB;
+    constexpr int B = MCM_EB;
     const int tot = d0 + d1;
     for (int o = 0; o < tot; o += B) {
       int v[B];
@@ -827,7 +858,7 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < B; k++) {
         const int x = o + k;
-        v[k] = x < d0 ? ld_ro(p.radj + s0 + x) : (x < tot ? ld_ro(p.radj + s1 + (x - d0)) : -1);
+        v[k] = x < d0 ? ld_adj(p.radj + s0 + x) : (x < tot ? ld_adj(p.radj + s1 + (x - d0)) : -1);
       }
 #pragma unroll
       for (int k = 0; k < B; k++) cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : ~0ull;
@@ -872,6 +903,7 @@ struct Solver {
   __device__ void gr_level_bu(int lvl, u32 base, int4 *next, u32 *ncnt, int *guard, u32 *gcnt) {
     const int lane = lane_id();
     const u32 lf = base + lvl, lc = base + lvl + 1, lr = base + lvl + 2;
+    int bt = 0;
     for (int t = cta<GRID>() * NT; t < n; t += ncta<GRID>() * NT) {
       const int v = t + (int)threadIdx.x;
       u64 cs = 0;
@@ -890,7 +922,7 @@ struct Solver {
           int x[KB];
           u64 rs[KB];
 #pragma unroll
-          for (int k = 0; k < KB; k++) x[k] = j + k < e ? ld_ro(p.cadj + j + k) : -1;
+          for (int k = 0; k < KB; k++) x[k] = j + k < e ? ld_adj(p.cadj + j + k) : -1;
 #pragma unroll
           for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
 #pragma unroll
@@ -909,7 +941,7 @@ struct Solver {
 #pragma unroll
           for (int k = 0; k < KB; k++) {
             const int jj = c0 + k * 32 + lane;
-            if (jj < eb) h |= psi_of(vld(p.rowst + ld_ro(p.cadj + jj))) == lf;
+            if (jj < eb) h |= psi_of(vld(p.rowst + ld_adj(p.cadj + jj))) == lf;
           }
           any = __any_sync(0xffffffffu, h);
           if (lane == 0) S(SS_GREDGES) += min(32 * KB, eb - c0);
@@ -932,8 +964,11 @@ struct Solver {
           if (w != -2) count_free();
         }
       }
-      flush(next, ncnt);
+      // every MCM_BUFLUSH tiles: a bottom-up level walks all n columns (C3: ~300
+      // tiles per CTA), so its output would overflow the shared staging
+      if (++bt % MCM_BUFLUSH == 0) flush(next, ncnt);
     }
+    flush(next, ncnt);
   }
   // bottom-up when the frontier's adjacency entries reach bu_div/8 times the
   // columns still unlabelled (Beamer-style edge rule; frontier rows alone mislead on
@@ -991,6 +1026,7 @@ struct Solver {
     g.nlen = (int)ring_prev(0);
     g.fedges = ring_prev(4);
     g.visited = (long long)g.nlen + ring_prev(2);
+    g.reached = (int)ring_prev(2);
     ulen = (int)ring_prev(1);
     int *tmp = U; U = T; T = tmp;
     g.lvl = 0; g.deepest = 0; g.cur_is_a = 1;
@@ -1164,37 +1200,44 @@ struct Solver {
         if (v >= 0) push_finalize(i, v, cs, best, ub, wb, loop, base, Ac, Ap);
         else if (i < len) Ap[i] = -1;                   // l.24
       }
-      __syncthreads();
-      // deferred long lists: with more than HUGE_CTA of them, those of at most
-      // HUGE_WARP entries get a warp each (in parallel), the rest the whole CTA each
-      // (a warp walks ~128 entries per round trip, the CTA ~2048: R-MAT hub columns
-      // of 10^5 entries on one warp held the phase for ~1.2 ms)
-      const int nh = min(sm.nhuge, MAXHUGE);
-      if (nh > HUGE_CTA) {
-        for (int h = warp_id(); h < nh; h += NWARP) {
-          const int4 hq = sm.huge[h];
-          if (hq.w - hq.z > HUGE_WARP) continue;
-          u64 hb;
-          int hu, hw;
-          scan(hq.z, hq.w, lane, 32, 0xffffffffu, sm.huget[h], base, hb, hu, hw);
-          if (lane == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
-        }
-      }
-      for (int h = 0; h < nh; h++) {
+    }
+    push_huge(loop, base, Ac, Ap);
+  }
+  // The columns a push phase deferred to the CTA (lists longer than HUGE_DEG, at most
+  // MAXHUGE per CTA and phase; beyond that the lane group / warp scans them itself):
+  // pushed once at the end of the phase, so the tiles of a phase never wait for each
+  // other.  With more than HUGE_CTA of them, those of at most HUGE_WARP entries get a
+  // warp each (in parallel), the rest the whole CTA each (a warp walks ~128 entries
+  // per round trip, the CTA ~2048: R-MAT hub columns of 10^5 entries on one warp held
+  // the phase for ~1.2 ms).  Publishes the CTA's dead-column count.
+  __device__ void push_huge(int loop, u32 base, int *Ac, int *Ap) {
+    const int lane = lane_id();
+    __syncthreads();
+    const int nh = min(sm.nhuge, MAXHUGE);
+    if (nh > HUGE_CTA) {
+      for (int h = warp_id(); h < nh; h += NWARP) {
         const int4 hq = sm.huge[h];
-        if (nh > HUGE_CTA && hq.w - hq.z <= HUGE_WARP) continue;
+        if (hq.w - hq.z > HUGE_WARP) continue;
         u64 hb;
         int hu, hw;
-        scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
-        if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+        scan(hq.z, hq.w, lane, 32, 0xffffffffu, sm.huget[h], base, hb, hu, hw);
+        if (lane == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
       }
-      __syncthreads();
-      if (threadIdx.x == 0) {
-        sm.nhuge = 0;
-        if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
-      }
-      __syncthreads();
     }
+    for (int h = 0; h < nh; h++) {
+      const int4 hq = sm.huge[h];
+      if (nh > HUGE_CTA && hq.w - hq.z <= HUGE_WARP) continue;
+      u64 hb;
+      int hu, hw;
+      scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
+      if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      sm.nhuge = 0;
+      if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
+    }
+    __syncthreads();
   }
   // PUSHKRNL on a wide worklist (more than two slots per thread): PB slots per
   // thread per tile, each stage's loads issued for all of them before any is used
@@ -1206,7 +1249,7 @@ struct Solver {
   // paths of push().
   template <bool GRID>
   __device__ void push_wide(int len, int *Ac, int *Ap, int loop, u32 base) {
-    constexpr int PB = 4;
+    constexpr int PB = MCM_PB;
     const int lane = lane_id();
     for (int t = cta<GRID>() * NT * PB; t < len; t += ncta<GRID>() * NT * PB) {
       int i[PB], v[PB], s[PB], e[PB], tg[PB];
@@ -1234,7 +1277,7 @@ struct Solver {
       for (int k = 0; k < PB; k++)
 #pragma unroll
         for (int q = 0; q < KB; q++)
-          x[k][q] = (v[k] >= 0 && e[k] - s[k] <= BIG_DEG && s[k] + q < e[k]) ? ld_ro(p.cadj + s[k] + q) : -1;
+          x[k][q] = (v[k] >= 0 && e[k] - s[k] <= BIG_DEG && s[k] + q < e[k]) ? ld_adj(p.cadj + s[k] + q) : -1;
 #pragma unroll
       for (int k = 0; k < PB; k++)
 #pragma unroll
@@ -1296,22 +1339,8 @@ struct Solver {
         if (v[k] >= 0) push_finalize(i[k], v[k], cs[k], best[k], ub[k], wb[k], loop, base, Ac, Ap, ia[k]);
         else if (v[k] == -1 && i[k] < len) Ap[i[k]] = -1;  // l.24
       }
-      __syncthreads();
-      const int nh = min(sm.nhuge, MAXHUGE);
-      for (int h = 0; h < nh; h++) {
-        const int4 hq = sm.huge[h];
-        u64 hb;
-        int hu, hw;
-        scan_cta(hq.z, hq.w, sm.huget[h], base, hb, hu, hw);
-        if (threadIdx.x == 0) push_finalize(hq.x, hq.y, sm.hugec[h], hb, hu, hw, loop, base, Ac, Ap);
-      }
-      __syncthreads();
-      if (threadIdx.x == 0) {
-        sm.nhuge = 0;
-        if (sm.nd) { atomicAdd(&p.ctrl->ndead, sm.nd); sm.nd = 0; }
-      }
-      __syncthreads();
     }
+    push_huge(loop, base, Ac, Ap);
   }
   // Push chains (single-CTA tail, at most chain_slots active columns; reading R26, a
   // build addition).  In the paper's loop a double push hands the displaced column
@@ -1436,7 +1465,7 @@ struct Solver {
 #pragma unroll
       for (int k = 0; k < KB; k++) {
         int jj = c0 + (int)threadIdx.x + k * NT;
-        x[k] = jj < e ? ld_ro(p.cadj + jj) : -1;
+        x[k] = jj < e ? ld_adj(p.cadj + jj) : -1;
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? vld(p.rowst + x[k]) : 0ull;
@@ -1495,7 +1524,7 @@ struct Solver {
         int jj = c0 + gl + k * G;
         int q = jj - s + rot;
         if (q >= len) q -= len;
-        x[k] = jj < e ? ld_ro(p.cadj + s + q) : -1;
+        x[k] = jj < e ? ld_adj(p.cadj + s + q) : -1;
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? (fresh ? ld_rlx(p.rowst + x[k]) : vld(p.rowst + x[k])) : 0ull;
@@ -1652,8 +1681,10 @@ struct Solver {
     long long loop, iterGR, gapAt;
     int len, ulen;
     u32 base;
-    int shrink, compact_next, gr_active, ac0, u0, pad;
+    int shrink, compact_next, gr_active, ac0, u0;
+    int cflags;            // concurrent GR (NEXT-2): bit 0 active, bit 1 the GR kernel's labels are ready
     int floor_r, floor_c;  // labels of vertices the last GR did not reach (m+n unless it stopped early)
+    u32 creq;              // concurrent GR (NEXT-2): requests sent to the GR kernel
     GRState gst;
   };
   static_assert(sizeof(Ctl) % 8 == 0 && sizeof(Ctl) / 8 <= 32, "Ctl handoff image");
@@ -1689,10 +1720,14 @@ struct Solver {
     if (threadIdx.x == 0) sm.qcnt = 0;
     __syncthreads();
   }
-  // call after the level's barrier; the overflow count is ring_prev(0)
+  // call after the level's barrier.  Everything the tail level produced is counted
+  // in shared memory (no L2 round trip after the tail's CTA barrier): sm.qcnt =
+  // staged rows (those beyond TQ went to the global queue, in order of the
+  // overflow counter), sm.lvc[0] = alive unmatched columns labelled (R22).
   __device__ void tail_sq_end(GRState &g, int4 *nxt_global, const int4 *nxt_shared) {
     sq = false;
-    const int ovf = (int)ring_prev(0), sc = min(sm.qcnt, TQ);
+    const int q = sm.qcnt, sc = min(q, TQ), ovf = q - sc;
+    const int rc = (int)sm.lvc[0];
     if (ovf == 0) {
       g.nlen = sc;
       g.in_smem = 1;
@@ -1701,8 +1736,10 @@ struct Solver {
       g.nlen = ovf + sc;
       g.in_smem = 0;
     }
+    g.reached += rc;
+    g.visited += rc;
     __syncthreads();
-    if (threadIdx.x == 0) sm.qcnt = 0;
+    if (threadIdx.x == 0) { sm.qcnt = 0; sm.lvc[0] = 0; }
     __syncthreads();
   }
   // a shared frontier must move to the global queue before the grid can see it
@@ -1730,6 +1767,10 @@ struct Solver {
     c.shrink = 1;
     c.gr_active = 0;
     c.base += stride();
+    if ((F & F_AUX) && (c.cflags & 1)) {  // NEXT-2: from now on the GR kernel relabels in the background
+      c.iterGR = 0x3fffffffffffffffLL;
+      conc_request(c);
+    }
   }
   // GR level 0 (INITRELABEL via the epoch bump + first expansion)
   template <bool GRID>
@@ -1748,7 +1789,6 @@ struct Solver {
     c.gr_active = 1;
     // early stop (R22): every alive unmatched column is active; stop once all of them
     // carry a label.  alive unmatched = n - matched - dead; matched = m - |U|.
-    c.gst.reached = (int)ring_prev(2);
     c.gst.target = early_gr() ? n - (m - n_iso - c.ulen) - (int)bcast_ld((const u32 *)&p.ctrl->ndead) : 0x7fffffff;
     if (p.gr_target < 1.0 && early_gr() && c.gst.target >= p.gr_target_min)  // R28
       c.gst.target = (int)ceil(p.gr_target * (double)c.gst.target);
@@ -1774,17 +1814,20 @@ struct Solver {
       gr_level_bu<GRID>(g.lvl, c.base, nxt, ring_now(0), nullptr, &p.ctrl->gcnt);
     else
       gr_level<GRID>(nullptr, cur, g.nlen, g.lvl, c.base, nxt, ring_now(0), nullptr, nullptr, nullptr, &p.ctrl->gcnt);
-    barrier<GRID>();
-    g.fedges = ring_prev(4);
-    if (smemq) {
+    if (smemq) {  // single-CTA tail: counts in shared memory, no ring read
+      barrier<GRID, false>();
+      g.fedges = 0;
       tail_sq_end(g, nxt, sfr(g.cur_is_a ? 1 : 0));
+      g.visited += g.nlen;
     } else {
+      barrier<GRID>();
+      g.fedges = ring_prev(4);
       g.nlen = (int)ring_prev(0);
       g.in_smem = 0;
+      g.reached += (int)ring_prev(2);
+      g.visited += (long long)g.nlen + ring_prev(2);
     }
     g.cur_is_a ^= 1;
-    g.reached += (int)ring_prev(2);
-    g.visited += (long long)g.nlen + ring_prev(2);
     if (g.nlen == 0) gr_finish(c);
     else if (g.reached >= g.target) gr_finish(c, true);
     if (GRID && MCM_FINE) tmark(106, 0);
@@ -1850,9 +1893,12 @@ struct Solver {
     } else {
       push<GRID>(c.len, Ac, Ap, lp, cur);
     }
-    if (chain_grid) {
+    const bool poll = GRID && (F & F_AUX) && (c.cflags & 1);  // NEXT-2: one grid-uniform look at the GR kernel
+    if (poll && lead()) st_rlx((int *)ring_now(6), ld_acq(&p.ctrl2->cdone) == c.creq ? 1 : 0);
+    if (chain_grid || poll) {
       barrier<GRID, true>();
-      adv = max(1, (int)ring_prev(5));
+      if (chain_grid) adv = max(1, (int)ring_prev(5));
+      if (poll && ring_prev(6)) c.cflags |= 2;
     } else {
       barrier<GRID, false>();
     }
@@ -1914,6 +1960,11 @@ struct Solver {
           continue;
         }
         if ((F & F_AUX) && p.mode == MODE_RELABEL && c.loop != c.iterGR) { reason = R_TERM; break; }  // GR done
+        if ((F & F_AUX) && (c.cflags & 1) && bcast_ld(&p.ctrl2->cdone) == c.creq) {  // NEXT-2: install on the grid
+          c.cflags |= 2;
+          reason = R_GRID;
+          break;
+        }
         if (c.loop == c.gapAt) { reason = R_GRID; break; }
         if (c.loop == c.iterGR) {
           if (c.ulen > up || base_overflow(c)) { reason = R_GRID; break; }
@@ -1988,7 +2039,7 @@ struct Solver {
         if (p.dead_skip && psiv >= INF) e = s;
         int psimin = INF, ub = -1, wb = -1;
         for (int j = s; j < e; j++) {
-          int x = ld_ro(p.cadj + j);
+          int x = ld_adj(p.cadj + j);
           u64 rs = vld(p.rowst + x);
           int l = labf(psi_of(rs), base, INF);
           S(SS_SCAN)++;
@@ -2158,6 +2209,10 @@ struct Solver {
 
   // ---------------------------------------------------------------- the solve
   __device__ __forceinline__ void run() {
+    if ((F & F_AUX) && p.mode == MODE_CONC_GR) {  // the GR kernel of a concurrent solve
+      conc_gr();
+      return;
+    }
     u64 t0 = tnow(), tA = t0;
     long long ns_init = 0;
     int *Ac = p.wl0, *Ap = p.wl1;
@@ -2169,7 +2224,10 @@ struct Solver {
     add_count(init_state(), 7);
     barrier<true>();
     if (ring_prev(7)) {  // a caller's array held an out-of-range entry
-      if (lead()) p.ctrl->err = -1;  // MCM_EINVAL
+      if (lead()) {
+        p.ctrl->err = -1;  // MCM_EINVAL
+        if ((F & F_AUX) && p.conc > 0) st_rlx((int *)&p.ctrl2->cexit, 1);  // release the GR kernel
+      }
       return;
     }
     if ((F & F_AUX) && p.mode == MODE_UNIT) {  // mcm_unit_step: one phase on the caller's state
@@ -2227,11 +2285,13 @@ struct Solver {
     memset(&c, 0, sizeof(c));
     c.len = len; c.ulen = ulen; c.base = 1; c.gapAt = -1; c.ac0 = 1; c.u0 = 1;  // loop = iterGR = 0
     c.floor_r = c.floor_c = INF;
+    c.cflags = ((F & F_AUX) && p.conc > 0 && p.mode == MODE_SOLVE) ? 1 : 0;
     for (;;) {
       if (c.loop >= p.max_loops) {
         if (lead()) p.ctrl->err = -5;
         break;
       }
+      if ((F & F_AUX) && (c.cflags & 2)) { conc_install(c); continue; }  // NEXT-2: the GR kernel's labels
       if ((F & F_SERIAL) && p.serial && !c.gr_active && c.loop != c.iterGR && c.loop != c.gapAt) {
         int r = serial_episode(c);
         if (r == R_CAP) {
@@ -2253,7 +2313,10 @@ struct Solver {
           if (lead()) p.ctrl->err = -5;
           break;
         }
-        if (r == R_TERM && !guard_step(c)) break;
+        if (r == R_TERM) {
+          if (F & F_AUX) conc_stop(c);
+          if (!guard_step(c)) break;
+        }
         continue;
       }
       // one unit of grid work
@@ -2274,8 +2337,12 @@ struct Solver {
         if (!first_step(c) && !guard_step(c)) break;
         continue;
       }
-      if (!loop_step<true>(c, Acp(c), App(c)) && !guard_step(c)) break;  // l.10-19 / termination
+      if (!loop_step<true>(c, Acp(c), App(c))) {                      // l.10-19 / termination
+        if (F & F_AUX) conc_stop(c);
+        if (!guard_step(c)) break;
+      }
     }
+    if (F & F_AUX) conc_stop(c);
     fixmatching(0, 1);                                                 // l.20
     barrier<true>();
     finish_stats(init_card, ns_init, (long long)(tnow() - tA));
@@ -2373,6 +2440,161 @@ struct Solver {
     }
     if (lead()) p.ctrl->stat[ST_MAXLEVEL] = r;
     barrier<true, false>();
+  }
+
+
+  // ---------------------------------------------------------------- concurrent GR (NEXT-2)
+  // The paper's future work: "concurrent execution of global-relabeling
+  // and push-relabel kernels".  With option gr_concurrent = A > 0 a solve is two
+  // co-resident persistent kernels on two streams: this GR kernel on A CTAs and the
+  // push kernel (run()) on the rest.  The GR kernel waits for a request, runs a
+  // complete level-synchronous BFS (Alg. 2 / 4-5 semantics) from the unmatched rows
+  // of the CURRENT matching -- which the push kernel keeps changing: the mates are
+  // read racily, so the labels describe a matching of a few loops ago -- into SHADOW
+  // label arrays (srow / scol, epoch-tagged like the packed words), publishes them,
+  // and waits again.  The push kernel keeps pushing on its installed labels and,
+  // at its next loop boundary after a completion, installs the shadow labels into
+  // the packed {mu, psi} words (pushes paused for that one pass) and requests the
+  // next GR.  Labels from a stale matching can be wrong (a column may look dead, a
+  // row may keep label 0 after it was matched): the exactness guard (R16) runs
+  // after termination as always, so the cardinality stays exact.
+  __device__ void conc_gr() {
+    Ctrl *x = p.ctrl;  // this kernel's own control block
+    const u32 sd = stride();
+    u32 sbase = 1, gen = 0;
+    int *Q[2] = {p.qc, p.qd};  // row frontiers (the push kernel uses qa / qb / wl0 / wl1)
+    const int GT = gridDim.x * NT, gt = blockIdx.x * NT + threadIdx.x;
+    int k = 0;  // level counter for the rotating frontier counters
+    auto gsync = [&](int j) {   // barrier; sm.rp[0] = ccnt[j] afterwards
+      grid_sync(&x->bar, false, [&] { sm.rp[0] = ld_rlx(&x->ccnt[j]); });
+    };
+    for (;;) {
+      if (threadIdx.x == 0) {
+        const u64 t0 = gtime();
+        u32 r;
+        for (;;) {
+          r = ld_acq(&x->creq);
+          if (r > gen || ld_rlx(&x->cexit)) break;
+          if (gtime() - t0 > 4000000000ull) { r = 0; break; }  // 4 s without a request: the push kernel is gone
+          __nanosleep(200);
+        }
+        sm.bc = (r > gen && !ld_rlx(&x->cexit)) ? r : 0u;
+      }
+      __syncthreads();
+      const u32 r = sm.bc;
+      __syncthreads();
+      if (r == 0) break;
+      gen = r;  // serve the latest request
+      if ((u64)sbase + 2ull * sd >= 0xfffffff0ull) {  // epoch overflow: all shadow labels stale again
+        for (int u = gt; u < m; u += GT) st_rlx((int *)p.srow + u, 0);
+        for (int v = gt; v < n; v += GT) st_rlx((int *)p.scol + v, 0);
+        gsync(0);
+        sbase = 1;
+      }
+      // level 0: the unmatched rows (with an edge) of the current matching, label 0
+      for (int t = blockIdx.x * NT; t < m; t += GT) {
+        const int u = t + (int)threadIdx.x;
+        bool f = false;
+        if (u < m && mu_of(vld(p.rowst + u)) == -1 && ld_ro(p.rptr + u) < ld_ro(p.rptr + u + 1)) {
+          st_rlx((int *)p.srow + u, (int)sbase);
+          f = true;
+        }
+        if (f) {
+          cg::coalesced_group g = cg::coalesced_threads();
+          u32 b = 0;
+          if (g.thread_rank() == 0) b = atomicAdd(&x->ccnt[k & 3], (u32)g.size());
+          Q[0][g.shfl(b, 0) + g.thread_rank()] = u;
+        }
+      }
+      gsync(k & 3);
+      int nlen = (int)sm.rp[0], cur = 0;
+      if (lead()) x->ccnt[(k + 2) & 3] = 0;
+      k++;
+      for (u32 lvl = 0; nlen > 0; lvl += 2) {
+        const u32 lc = sbase + lvl + 1, lr = sbase + lvl + 2;
+        constexpr int GL = 8;  // lanes per frontier row
+        const int gl = lane_id() & (GL - 1);
+        for (int t = blockIdx.x * (NT / GL); t < nlen; t += gridDim.x * (NT / GL)) {
+          const int i = t + (int)threadIdx.x / GL;
+          const int u = i < nlen ? __ldcg(Q[cur] + i) : -1;
+          const int s0 = u >= 0 ? ld_ro(p.rptr + u) : 0, e0 = u >= 0 ? ld_ro(p.rptr + u + 1) : 0;
+          for (int j = s0 + gl; j < e0; j += GL) {
+            const int v = ld_adj(p.radj + j);
+            const u32 sv = (u32)ld_rlx((const int *)p.scol + v);
+            if (sv >= sbase || atomicCAS(p.scol + v, sv, lc) != sv) continue;  // visited, or claimed by another
+            const int w = mu_of(vld(p.colst + v));
+            if (w < 0 || mu_of(vld(p.rowst + w)) != v) continue;  // not matched (Alg. 5 l.6)
+            st_rlx((int *)p.srow + w, (int)lr);
+            cg::coalesced_group g = cg::coalesced_threads();
+            u32 b = 0;
+            if (g.thread_rank() == 0) b = atomicAdd(&x->ccnt[k & 3], (u32)g.size());
+            Q[cur ^ 1][g.shfl(b, 0) + g.thread_rank()] = w;
+          }
+        }
+        gsync(k & 3);
+        nlen = (int)sm.rp[0];
+        if (lead()) x->ccnt[(k + 2) & 3] = 0;
+        k++;
+        cur ^= 1;
+      }
+      // every CTA passed the last barrier: the labels are complete -> publish
+      if (lead()) {
+        for (int j = 0; j < 4; j++) x->ccnt[j] = 0;
+        st_rlx((int *)&x->csbase, (int)sbase);
+        __threadfence();
+        asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(&x->cdone), "r"(gen) : "memory");
+        L().grs++;
+      }
+      k = 0;
+      sbase += sd;
+      gsync(0);  // the counters are zero before anyone appends again
+    }
+    grid_sync(&x->bar, false);
+    if (lead()) asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(&x->cexited), "r"(1u) : "memory");
+  }
+  // push kernel: the GR kernel finished the requested labels (CTA-uniform via sm.bc)
+  __device__ bool conc_ready(const Ctl &c) {
+    return (c.cflags & 1) && bcast_ld(&p.ctrl2->cdone) == c.creq;
+  }
+  __device__ void conc_request(Ctl &c) {
+    c.creq++;
+    if (lead()) asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(&p.ctrl2->creq), "r"(c.creq) : "memory");
+  }
+  // install the shadow labels into the packed words (every push-kernel CTA, pushes
+  // paused at a loop boundary), move to the new epoch, request the next GR
+  __device__ void conc_install(Ctl &c) {
+    u64 g0 = tnow();
+    const u32 sb = bcast_ld(&p.ctrl2->csbase);
+    if (base_overflow(c)) { reset_labels(); c.base = 1; }
+    const u32 nb = c.base;
+    const int G = gridDim.x * NT, g = blockIdx.x * NT + threadIdx.x;
+    for (int u = g; u < m; u += G) {
+      const u32 sl = (u32)ld_rlx((const int *)p.srow + u);
+      if (sl >= sb) vst(p.rowst + u, pack(mu_of(vld(p.rowst + u)), nb + (sl - sb)));
+    }
+    for (int v = g; v < n; v += G) {
+      const u32 sl = (u32)ld_rlx((const int *)p.scol + v);
+      if (sl >= sb) vst(p.colst + v, pack(mu_of(vld(p.colst + v)), nb + (sl - sb)));
+    }
+    barrier<true, false>();
+    c.base += stride();
+    c.floor_r = c.floor_c = INF;
+    c.cflags &= ~2;
+    c.shrink = 1;  // Alg. 7 l.9: the worklist is compacted after a GR
+    if (lead()) { L().grs++; L().ns_gr += (long long)(tnow() - g0); }
+    conc_request(c);
+  }
+  // stop the GR kernel (it finishes a running BFS first) before the queues it uses
+  // are needed again (guard GR) or the solve ends
+  __device__ void conc_stop(Ctl &c) {
+    if (!(c.cflags & 1)) return;
+    if (lead()) {
+      asm volatile("st.release.gpu.global.u32 [%0], %1;" ::"l"(&p.ctrl2->cexit), "r"(1u) : "memory");
+      const u64 t0 = gtime();
+      while (!ld_acq(&p.ctrl2->cexited) && gtime() - t0 < 8000000000ull) __nanosleep(200);
+    }
+    barrier<true, false>();
+    c.cflags = 0;
   }
 
   __device__ void reset_labels() {

@@ -1,7 +1,7 @@
 """Repeat small solves and report any invalid matching in detail (GPU box):
 
-    python tools/race_repro.py [reps] [graph] [opt=val,...]
-    compute-sanitizer --tool racecheck python tools/race_repro.py 1 C2
+    python tests/race_repro.py [reps] [graph] [opt=val,...]
+    compute-sanitizer --tool racecheck python tests/race_repro.py 1 C2
 
 graph: C2 (C2 at scale 0.002, default), C1, hall.  On an invalid result it prints
 the check code, the conflicting rows / columns and the solve statistics.

@@ -1,8 +1,8 @@
 """Small solves for compute-sanitizer runs (GPU box):
 
-    compute-sanitizer --tool memcheck python tools/sanitize.py
-    compute-sanitizer --tool synccheck python tools/sanitize.py
-    compute-sanitizer --tool racecheck python tools/sanitize.py quick
+    compute-sanitizer --tool memcheck python tests/sanitize_solves.py
+    compute-sanitizer --tool synccheck python tests/sanitize_solves.py
+    compute-sanitizer --tool racecheck python tests/sanitize_solves.py quick
 
 Every solve goes through the C ABI (create, solve, relabel entries, host-buffer
 entry) on graphs small enough for the instrumented kernel, covering the grid
@@ -46,6 +46,22 @@ def main():
     run(g, gap=1)
     run(g, variant=1)
     run(g, tail_chain=0, grid_chain=0, gr_early=0, compact_adapt=0)
+    run(g, gr_concurrent=32)
+    # round-2 entry points: the device M0, a GR through the tail, one phase of each kind
+    ip, ix = torch.from_numpy(g.indptr).cuda(), torch.from_numpy(g.indices).cuda()
+    mt = pkg.Matcher(ip, ix, g.m, g.n, sort_csc=1)
+    c0, rm, cm = mt.initial_matching()
+    assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == c0
+    ml, pr, pc, rf = mt.global_relabel(rm, cm)
+    INF = g.m + g.n
+    for unit in ("fix", "shrink", "push", "fixmatching"):
+        for where in ("grid", "tail"):
+            st = [rm.clone(), cm.clone(), pr.clone(), pc.clone(), torch.full((g.n,), -1, dtype=torch.int32, device="cuda"),
+                  torch.arange(min(g.n, 300), dtype=torch.int32, device="cuda"),
+                  torch.full((min(g.n, 300),), -1, dtype=torch.int32, device="cuda")]
+            mt.unit_step(unit, where, 3, *st)
+    mt.close()
+    print("unit / relabel / initial-matching entries ok", c0, ml, INF)
     # host-buffer entry
     g = synth.config("C5", 1 / 1024, index=1)
     card, rm, cm, _ = pkg.match_host(torch.from_numpy(g.indptr).pin_memory(), torch.from_numpy(g.indices).pin_memory(),

@@ -117,6 +117,8 @@ OPTION_SETS = [
     dict(grid_chain=1), dict(grid_chain=1 << 30), dict(grid_chain=4, tail_max=0), dict(grid_chain=0, tail_chain=0),
     dict(grid_chain=1000, tail_max=0, k=0.1), dict(gr_target=1.0), dict(gr_target=0.8, gr_target_min=0),
     dict(gr_target=0.3, k=0.3, gr_target_min=0), dict(gr_target=0.01, tail_max=0, gr_target_min=16),
+    dict(gr_concurrent=48), dict(gr_concurrent=16, k=3.0), dict(gr_concurrent=100, tail_max=0),
+    dict(gr_concurrent=1, grid_chain=0, tail_chain=0),
 ]
 
 
@@ -388,3 +390,26 @@ def test_serial_mode_matches_simulator(ci):
                shrinks=gst["shrinks"], dead=gst["dead"], blocked=gst["blocked"], gaps=gst["gaps"])
     want = {k: st[k] for k in got}
     assert got == want, (g.name, kw, got, want)
+
+
+def test_concurrent_gr_repeated():
+    """NEXT-2 (gr_concurrent): the GR kernel and the push kernel race on the matching
+    by design; repeated solves stay exact (the guard) and the GR kernel is always
+    released (no solve hangs), also after a rejected input."""
+    g = synth.config("C2", 0.05)
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, gr_concurrent=48)
+    for _ in range(10):
+        card, rm, cm = mt.solve()
+        assert card == g.n
+        assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == card
+    mt.close()
+    _, rm0, cm0 = oracle.cheap_match(g)
+    bad = rm0.astype(np.int32).copy()
+    bad[0] = g.n  # out of range: MCM_EINVAL, the GR kernel must still exit
+    mt = pkg.Matcher(ip, ix, g.m, g.n, gr_concurrent=48, init="given")
+    with pytest.raises(pkg.MCMError):
+        mt.solve(torch.from_numpy(bad).to(DEV), torch.from_numpy(cm0.astype(np.int32)).to(DEV))
+    card, _, _ = mt.solve(torch.from_numpy(rm0.astype(np.int32)).to(DEV), torch.from_numpy(cm0.astype(np.int32)).to(DEV))
+    assert card == g.n
+    mt.close()

@@ -29,9 +29,11 @@ METRICS = [
 
 
 def launches(tag):
-    path = os.path.join(OUT, "launches_C2.csv")
-    if not os.path.exists(path):
-        return
+    for path in sorted(glob.glob(os.path.join(OUT, "launches_*.csv"))):
+        launches_one(tag, path, os.path.basename(path)[9:-4])
+
+
+def launches_one(tag, path, cfg):
     lines = [ln for ln in open(path) if not ln.startswith("==")]
     rows = list(csv.DictReader(io.StringIO("".join(lines))))
     agg = defaultdict(lambda: [0, 0.0])
@@ -42,8 +44,8 @@ def launches(tag):
         agg[r["Kernel Name"]][0] += 1
         agg[r["Kernel Name"]][1] += us
     tot = sum(v[1] for v in agg.values())
-    with open(os.path.join(PROF, f"{tag}_launches_C2.md"), "w") as f:
-        f.write(f"# {tag}: ncu launch list of `python bench.py --steps 2 --warmup 3 --no-cpu-baseline` (C2)\n\n")
+    with open(os.path.join(PROF, f"{tag}_launches_{cfg}.md"), "w") as f:
+        f.write(f"# {tag}: ncu launch list of `python bench.py --config {cfg} --steps 2 --warmup 3 --no-cpu-baseline`\n\n")
         f.write("`ncu --metrics gpu__time_duration.sum --clock-control none -c 400` -- cold-cache, serialised "
                 "per-launch times: compare SHARES, not absolutes.\n\n")
         f.write("| kernel | launches | total us | mean us | share |\n|---|---|---|---|---|\n")
