@@ -147,6 +147,15 @@ typedef struct {
                            pushing; finished labels are installed at the next loop boundary.
                            The exactness guard keeps the result exact.  Ignored in serial mode
                            and for G-PR-First.  Default 0 (off). */
+  int32_t perturb;      /* fault injection (tests only): each of the paper's
+                           pushes (Alg. 9 l.14-18, not the push chains of R26) loses its row
+                           store with probability perturb / 65536 (a counter hash of the
+                           column and the loop): mu(v) <- u and Ap(i) <- w are written, the
+                           row word keeps its old mate -- the outcome of losing the race for
+                           u to another column.  The column is then active by
+                           reading R1 and is pushed again; the rollback (Alg. 8 l.3-6),
+                           FIXMATCHING and the exactness guard must still return
+                           a maximum matching.  0..65536; default 0 (off). */
 } mcm_options_t;
 
 typedef struct {
@@ -282,6 +291,40 @@ int64_t mcm_unit_step(mcm_handle_t h, mcm_stream_t stream, int32_t unit, int32_t
  * is no gap, or a negative error code below -1.  This is the same device routine
  * the solve applies once between two GRs when options.gap = 1. */
 int64_t mcm_gap_relabel(mcm_handle_t h, mcm_stream_t stream, int32_t *psi_row, int32_t *psi_col);
+
+/* ---- NEXT-4 (an EXPERIMENT, not on the solve path) ----
+ * A 1D row-partitioned global relabel (Alg. 2 with the matched test of Alg. 5 l.6,
+ * P:257-272, 401-410) whose BFS levels exchange the row frontier as a bitmap with
+ * an all-gather (NCCL over NVLink in paper_conf_icpp_devecikuc13_b200/pgr.py).  It
+ * exists to measure why replicas win: one collective per BFS level.
+ *   nparts P >= 1 parts, this call's part p (0 <= p < P), words W >= 1 bitmap words
+ *   (32 rows each) per part, with 32 W P >= m.  Part p owns rows [32 W p, 32 W (p+1))
+ *   and the mate column of each owned row u with cmatch[rmatch[u]] = u (the column
+ *   is matched, Alg. 5 l.6), plus the columns that are not matched in
+ *   [ceil(n/P) p, ceil(n/P) (p+1)).
+ *   Frontier buffers (DEVICE uint32): P slices of W + 1 words, part q's slice at
+ *   word q (W + 1): W bitmap words (bit u mod 32 of word (u mod 32W) / 32 = row u
+ *   is in the frontier) and one count word (rows the part added).  `slice` points
+ *   at THIS part's slice (W + 1 words) of the buffer being built, `frontier` at the
+ *   whole gathered buffer of the previous level.
+ *   psi_row (m) / psi_col (n): DEVICE int32 labels; only owned entries are written
+ *   after mcm_pgr_init (the elementwise minimum over the parts is the GR result:
+ *   the exact BFS distance, m+n when unreached).  rmatch (m) / cmatch
+ *   (n): DEVICE, the matching with the paper's mu conventions (cmatch may be stale
+ *   or -2; rows are authoritative); entries out of range are treated as unmatched.
+ * Both calls only enqueue work on `stream` (no synchronisation) and return MCM_OK
+ * or a negative error code. */
+/* Level 0 (Alg. 2 l.1-3): owned rows get 0 (unmatched) or m+n, every column m+n;
+ * writes this part's slice of F_0. */
+int mcm_pgr_init(mcm_handle_t h, mcm_stream_t stream, int32_t nparts, int32_t part, int32_t words,
+                 const int32_t *rmatch, uint32_t *slice, int32_t *psi_row, int32_t *psi_col);
+/* Level L >= 0 (row labels 2L form `frontier`): every unlabelled owned column v
+ * with a row of Gamma(v) in the frontier gets 2L+1, its owned mate row 2L+2 (the
+ * row joins this part's slice of F_{L+1}).  *reached_free (DEVICE uint64,
+ * accumulated) += columns that are not matched and got a label. */
+int mcm_pgr_level(mcm_handle_t h, mcm_stream_t stream, int32_t nparts, int32_t part, int32_t words, int32_t level,
+                  const int32_t *rmatch, const int32_t *cmatch, const uint32_t *frontier, uint32_t *slice,
+                  int32_t *psi_row, int32_t *psi_col, uint64_t *reached_free);
 
 /* Replace the options of a handle (takes effect at the next solve). */
 int mcm_set_options(mcm_handle_t h, const mcm_options_t *o);

@@ -64,6 +64,7 @@ class Options(ctypes.Structure):
         ("gr_target", ctypes.c_double),
         ("gr_target_min", ctypes.c_int32),
         ("gr_concurrent", ctypes.c_int32),
+        ("perturb", ctypes.c_int32),
     ]
 
 
@@ -117,6 +118,10 @@ def lib():
         L.mcm_unit_step.restype = i64
         L.mcm_gap_relabel.argtypes = [vp, vp, vp, vp]
         L.mcm_gap_relabel.restype = i64
+        L.mcm_pgr_init.argtypes = [vp, vp, i32, i32, i32, vp, vp, vp, vp]
+        L.mcm_pgr_init.restype = ctypes.c_int
+        L.mcm_pgr_level.argtypes = [vp, vp, i32, i32, i32, i32, vp, vp, vp, vp, vp, vp, vp]
+        L.mcm_pgr_level.restype = ctypes.c_int
         L.mcm_set_options.argtypes = [vp, P(Options)]
         L.mcm_set_options.restype = ctypes.c_int
         L.mcm_set_k.argtypes = [vp, ctypes.c_double]
@@ -291,6 +296,31 @@ class Matcher:
         if g < -1:
             raise MCMError(int(g), "mcm_gap_relabel")
         return int(g), pr, pc
+
+    # NEXT-4 experiment (include/mcm.h mcm_pgr_*; orchestration in pgr.py)
+    def pgr_init(self, nparts, part, words, rmatch, slice_, psi_row, psi_col, stream=None):
+        torch = _torch()
+        with torch.cuda.device(self.device):
+            rc = lib().mcm_pgr_init(self._h, _stream_ptr(stream), nparts, part, words,
+                                    _dev_i32(rmatch, "rmatch", self.m), _dev_i32(slice_, "slice", words + 1),
+                                    _dev_i32(psi_row, "psi_row", self.m), _dev_i32(psi_col, "psi_col", self.n))
+        if rc != MCM_OK:
+            raise MCMError(rc, "mcm_pgr_init")
+
+    def pgr_level(self, nparts, part, words, level, rmatch, cmatch, frontier, slice_, psi_row, psi_col,
+                  reached_free, stream=None):
+        torch = _torch()
+        if not (isinstance(reached_free, torch.Tensor) and reached_free.is_cuda and reached_free.dtype == torch.int64
+                and reached_free.numel() == 1):
+            raise TypeError("reached_free must be a CUDA int64 tensor of 1 element")
+        with torch.cuda.device(self.device):
+            rc = lib().mcm_pgr_level(self._h, _stream_ptr(stream), nparts, part, words, level,
+                                     _dev_i32(rmatch, "rmatch", self.m), _dev_i32(cmatch, "cmatch", self.n),
+                                     _dev_i32(frontier, "frontier", nparts * (words + 1)),
+                                     _dev_i32(slice_, "slice", words + 1), _dev_i32(psi_row, "psi_row", self.m),
+                                     _dev_i32(psi_col, "psi_col", self.n), ctypes.c_void_p(reached_free.data_ptr()))
+        if rc != MCM_OK:
+            raise MCMError(rc, "mcm_pgr_level")
 
     def stats(self) -> dict:
         s = Stats()

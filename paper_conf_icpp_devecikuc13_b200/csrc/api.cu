@@ -1,6 +1,7 @@
 // api.cu -- the C ABI of include/mcm.h: workspace layout, graph ingest (validate,
 // copy, CSC transpose) and the cooperative launch of the persistent G-PR kernel.
 #include <cuda_runtime.h>
+#include <nvtx3/nvToolsExt.h>
 #include <chrono>
 #include <cmath>
 #include <cstdio>
@@ -10,6 +11,16 @@
 #include <memory>
 #include <algorithm>
 #include <vector>
+
+// NVTX ranges (SURVEY.md 5 "tracing"): one per host-visible step of the path
+// (validation + copy, CSC transpose, each kernel launch by mode, host copies);
+// the phases inside the persistent kernel are traced by MCM_TRACE instead.
+struct NvtxRange {
+  explicit NvtxRange(const char *name) { nvtxRangePushA(name); }
+  ~NvtxRange() { nvtxRangePop(); }
+  NvtxRange(const NvtxRange &) = delete;
+  NvtxRange &operator=(const NvtxRange &) = delete;
+};
 
 #include "../../include/mcm.h"
 #include "solve.cuh"
@@ -289,6 +300,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->tail_ctas < 1 || o->tail_ctas > 16 || (o->tail_ctas & (o->tail_ctas - 1))) return MCM_EINVAL;
   if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0 || o->grid_chain < 0) return MCM_EINVAL;
   if (o->gr_concurrent < 0 || o->gr_concurrent > MAX_CTAS) return MCM_EINVAL;
+  if (o->perturb < 0 || o->perturb > 65536) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -304,6 +316,7 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
   Layout L = layout(m, n, nnz);
   if (ws_bytes < L.total) return MCM_ENOMEM;
   cudaStream_t st = (cudaStream_t)stream_;
+  NvtxRange r_create(from_host ? "mcm_create(host CSR)" : "mcm_create");
   auto t0 = std::chrono::steady_clock::now();
   h = new (std::nothrow) mcm_ctx();
   if (!h) return MCM_ENOMEM;
@@ -342,6 +355,7 @@ static int create_impl(const int32_t *indptr, const int32_t *indices, int32_t m,
   if (herr) return MCM_EINVAL;
 
   int *cptr = (int *)(ws + L.cptr), *cadj = (int *)(ws + L.cadj);
+  NvtxRange r_csc("mcm_create: CSC transpose");
   // CSC by counting sort (Gamma(v) for the push, Alg. 9 l.6): degrees
   // (k_ingest), exclusive scan, scatter.  (Rejected alternatives, measured: a
   // pass-blocked scatter keeping each pass's cadj segment in L2, 5.3 ms on C4, round
@@ -397,6 +411,9 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
                       int32_t *out_c, int32_t *host_r = nullptr, int32_t *host_c = nullptr,
                       const UnitArgs *ua = nullptr) {
   if (h->poisoned) return MCM_ECUDA;
+  static const char *const mode_name[] = {"mcm_solve", "mcm_global_relabel", "mcm_gap_relabel", "mcm_unit_step",
+                                          "mcm_initial_matching", "mcm_solve"};
+  NvtxRange r_launch(mode_name[mode >= 0 && mode <= MODE_CONC_GR ? mode : 0]);
   int dev = -1;
   CK(cudaGetDevice(&dev));
   if (dev != h->dev) return MCM_EDEVICE;
@@ -438,6 +455,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.serial = o.serial;
   p.variant = o.variant;
   p.tail_chain = o.tail_chain;
+  p.perturb = o.perturb;
   // worklists of at most this many slots run as push chains (lanes per slot from the
   // count); MCM_CHAIN_SLOTS: analysis knob
   // (analysis knobs, clamped: 0..TW slots; a divisor of at least 1)
@@ -473,7 +491,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   // the lean production instance unless a feature only the full one carries is on
   // (a cluster tail group spans several SMs' L1s: it needs gpu-scope vertex state)
   const bool conc = mode == MODE_SOLVE && o.gr_concurrent > 0 && !o.serial && !o.variant;
-  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1 || conc)
+  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1 || conc || o.perturb)
                                    ? gpr_kernel<F_ALL>
                                    : gpr_kernel<F_FAST>;
   if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
@@ -593,6 +611,7 @@ int64_t mcm_match_host(const int32_t *indptr, const int32_t *indices, int32_t m,
                        int32_t *cmatch, mcm_stats_t *stats) {
   if ((m > 0 && !rmatch) || (n > 0 && !cmatch)) return MCM_EINVAL;
   if (o && o->init == MCM_INIT_GIVEN) return MCM_EINVAL;  // no device copy of a given matching on this path
+  NvtxRange r_e2e("mcm_match_host");
   mcm_handle_t h = nullptr;
   int rc = create_impl(indptr, indices, m, n, nnz, workspace, ws_bytes, stream, o, &h, true);
   if (rc != MCM_OK) return rc;
@@ -631,6 +650,54 @@ int64_t mcm_unit_step(mcm_handle_t h, mcm_stream_t stream, int32_t unit, int32_t
     return MCM_EINVAL;
   UnitArgs ua{unit, where, len, loop, psi_row, psi_col, iA, Ac, Ap};
   return launch(h, (cudaStream_t)stream, MODE_UNIT, mu_row, mu_col, mu_row, mu_col, nullptr, nullptr, &ua);
+}
+
+// NEXT-4 experiment (pgr.cu): partitioned GR levels on the handle's CSC
+int mcm_internal_pgr_init(int m, int n, int P, int p, int W, const int *rmatch, uint32_t *slice, int *psi_row,
+                          int *psi_col, cudaStream_t st);
+int mcm_internal_pgr_level(int m, int n, int P, int p, int W, int L, const int *cptr, const int *cadj,
+                           const int *rmatch, const int *cmatch, const uint32_t *F, uint32_t *slice, int *psi_row,
+                           int *psi_col, unsigned long long *counts, cudaStream_t st);
+
+static bool pgr_args_ok(const mcm_ctx *h, int32_t nparts, int32_t part, int32_t words) {
+  if (nparts < 1 || part < 0 || part >= nparts || words < 1) return false;
+  return (int64_t)words * 32 * nparts >= h->m && (int64_t)words * nparts * 33 < ((int64_t)1 << 31);
+}
+
+int mcm_pgr_init(mcm_handle_t h, mcm_stream_t stream, int32_t nparts, int32_t part, int32_t words,
+                 const int32_t *rmatch, uint32_t *slice, int32_t *psi_row, int32_t *psi_col) {
+  if (!h || !pgr_args_ok(h, nparts, part, words) || !slice || (h->m > 0 && (!rmatch || !psi_row)) ||
+      (h->n > 0 && !psi_col))
+    return MCM_EINVAL;
+  if (h->poisoned) return MCM_ECUDA;
+  NvtxRange r("mcm_pgr_init");
+  if (int rc = mcm_internal_pgr_init(h->m, h->n, nparts, part, words, rmatch, slice, psi_row, psi_col,
+                                     (cudaStream_t)stream)) {
+    h->poisoned = true;
+    last_cuda_error = (cudaError_t)rc;
+    return MCM_ECUDA;
+  }
+  return MCM_OK;
+}
+
+int mcm_pgr_level(mcm_handle_t h, mcm_stream_t stream, int32_t nparts, int32_t part, int32_t words, int32_t level,
+                  const int32_t *rmatch, const int32_t *cmatch, const uint32_t *frontier, uint32_t *slice,
+                  int32_t *psi_row, int32_t *psi_col, uint64_t *reached_free) {
+  if (!h || !pgr_args_ok(h, nparts, part, words) || !frontier || !slice || !reached_free || level < 0 ||
+      2LL * level + 2 >= (int64_t)h->m + h->n + 2 || (h->m > 0 && (!rmatch || !psi_row)) ||
+      (h->n > 0 && (!cmatch || !psi_col)))
+    return MCM_EINVAL;
+  if (h->poisoned) return MCM_ECUDA;
+  NvtxRange r("mcm_pgr_level");
+  const Layout &L = h->L;
+  if (int rc = mcm_internal_pgr_level(h->m, h->n, nparts, part, words, level, (const int *)(h->ws + L.cptr),
+                             (const int *)(h->ws + L.cadj), rmatch, cmatch, frontier, slice, psi_row, psi_col,
+                             (unsigned long long *)reached_free, (cudaStream_t)stream)) {
+    h->poisoned = true;
+    last_cuda_error = (cudaError_t)rc;
+    return MCM_ECUDA;
+  }
+  return MCM_OK;
 }
 
 int64_t mcm_gap_relabel(mcm_handle_t h, mcm_stream_t stream, int32_t *psi_row, int32_t *psi_col) {

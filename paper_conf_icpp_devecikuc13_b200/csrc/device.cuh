@@ -43,6 +43,12 @@ __device__ __forceinline__ void st_rlx(int *p, int v) {
 }
 // read-only graph arrays (never written during a solve)
 __device__ __forceinline__ int ld_ro(const int *p) { return __ldg(p); }
+// counter hash of two words (fault injection, option perturb)
+__device__ __forceinline__ u32 hash2(u32 a, u32 b) {
+  u32 x = a * 0x9E3779B1u ^ (b + 0x7F4A7C15u) * 0x85EBCA77u;
+  x ^= x >> 15; x *= 0x2C1B3C6Du; x ^= x >> 12; x *= 0x297A2D39u; x ^= x >> 15;
+  return x;
+}
 // adjacency lists (radj / cadj): streamed, read-only.  (L2 evict_first hints on
 // these, and evict_last on the vertex state, were measured in round 2: within
 // noise on C2-C5, profiles/r02_l2hint_ab.txt; not kept.)

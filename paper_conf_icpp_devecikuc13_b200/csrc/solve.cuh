@@ -119,6 +119,7 @@ struct Params {
   int grid_chain_div;
   int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
   int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
+  int perturb;             // fault injection: a push loses its row store with probability perturb/65536
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -1131,7 +1132,11 @@ struct Solver {
     int psimin = best == ~0ull ? INF : (int)(best >> 32);
     if (psimin < INF) {                                 // l.12
       if (wb == -1 || (iaw == IA_LOAD ? vld(p.iA + wb) : iaw) != loop) {  // l.13
-        vst(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
+        // option perturb (F_AUX builds only): the row store is lost, as if another
+        // column had won the race for ub; v stays active by R1
+        if (!((F & F_AUX) && p.perturb &&
+              (hash2((u32)v, (u32)loop) & 0xffffu) < (u32)p.perturb))
+          vst(p.rowst + ub, pack(v, base + (u32)psimin + 2u));  // l.14, l.17
         vst(p.colst + v, pack(ub, base + (u32)psimin + 1u));  // l.15, l.16
         Ap[i] = wb;                                     // l.18 (R3)
         S(SS_PUSH)++;

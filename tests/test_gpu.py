@@ -172,6 +172,32 @@ def test_stale_rows_repaired(drop_cols, final_check):
         assert oracle.konig_cover(g, rm, cm)[0] == card
 
 
+@pytest.mark.parametrize("rate", [2048, 16384, 49152])
+@pytest.mark.parametrize("chains", [0, 1])
+def test_perturb_fault_injection(rate, chains):
+    """SURVEY.md 5 fault injection: option perturb drops the row store of a share of
+    the paper's pushes (the state a lost race for the row leaves).  The
+    column stays active by reading R1 and is pushed again; the solve must still
+    return a valid maximum matching with a Koenig certificate.  With a high rate the
+    paper's pushes need several tries, so the push count exceeds the unperturbed one."""
+    extra = {} if chains else dict(grid_chain=0, tail_chain=0)
+    for g in (synth.config("C1", 0.5), synth.config("C2", 0.005), synth.hall_violator(3000, 150, 41, 9)):
+        _, st0 = check_solve(g, **extra)
+        _, st = check_solve(g, perturb=rate, **extra)
+        if rate >= 16384 and not chains:
+            assert st["pushes"] > st0["pushes"], (g.name, st0["pushes"], st["pushes"])
+
+
+def test_perturb_without_guard_is_valid():
+    """perturb with the exactness guard off: FIXMATCHING (R15) still
+    reports a valid matching (rows are authoritative)."""
+    g = synth.config("C2", 0.005)
+    ip, ix = dev(g)
+    mt = pkg.Matcher(ip, ix, g.m, g.n, perturb=16384, final_check=0, grid_chain=0, tail_chain=0)
+    card, rm, cm = mt.solve()
+    assert oracle.check_matching(g, rm.cpu().numpy(), cm.cpu().numpy()) == card
+
+
 def test_edge_cases():
     check_solve(synth.from_pairs(0, 0, [], []), 0)
     check_solve(synth.from_pairs(5, 0, [], []), 0)

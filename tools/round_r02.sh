@@ -3,8 +3,8 @@
 #   smoke, GPU tests, bench lines (C4 default; C1/C2/C3/C5, all with cpu_baseline),
 #   ncu launch list of the default bench command, one `ncu --set full` capture of
 #   the solve kernel on C4 and C2, phase traces, Fig. 1 (paper and build
-#   configurations on C2-C4), compute-sanitizer memcheck / racecheck.
-#   Skip parts with NOTESTS=1, NOFIG=1, NOSAN=1, NONCU=1.
+#   configurations on C2-C4), NEXT-4 partitioned-GR experiment.
+#   Skip parts with NOTESTS=1, NOFIG=1, NOPGR=1, NONCU=1.
 set -u
 O=gpurun_out
 T=${TAG:-r02}
@@ -30,7 +30,5 @@ if [ -z "${NOFIG:-}" ]; then
   timeout 1200 python tools/fig1.py paper C2 C3 C4 > $O/${T}_fig1_paper.md 2> $O/${T}_fig1_paper.err
   timeout 1200 python tools/fig1.py build C2 C3 C4 > $O/${T}_fig1_build.md 2> $O/${T}_fig1_build.err
 fi
-if [ -z "${NOSAN:-}" ]; then
-  timeout 600 compute-sanitizer --tool memcheck python tests/sanitize_solves.py quick > $O/${T}_san_memcheck.log 2>&1; echo "memcheck rc=$?" >> $O/${T}_san_rc.txt
-  timeout 900 compute-sanitizer --tool racecheck python tests/sanitize_solves.py quick > $O/${T}_san_racecheck.log 2>&1; echo "racecheck rc=$?" >> $O/${T}_san_rc.txt
-fi
+# (compute-sanitizer is closed on the GPU pool: not run)
+[ -z "${NOPGR:-}" ] && timeout 900 python tools/pgr_experiment.py C2 C3 C4 > $O/${T}_pgr.md 2> $O/${T}_pgr.err
