@@ -156,6 +156,14 @@ typedef struct {
                            reading R1 and is pushed again; the rollback (Alg. 8 l.3-6),
                            FIXMATCHING and the exactness guard must still return
                            a maximum matching.  0..65536; default 0 (off). */
+  int32_t gr_window;    /* windowed GR levels (a build addition; the paper's GR is level-synchronous,
+                           Alg. 5): K > 1 = every CTA expands its share of a grid
+                           frontier and the rows that share reaches, K levels deep, before the
+                           next grid barrier; labels are lowered by CAS (label correcting), so
+                           every label is the exact BFS distance at the window's end (DESIGN.md
+                           R29).  0 or 1 = one level per barrier.  0..64 */
+  int32_t gr_window_max; /* windows run for grid frontiers of at most this many rows (wider
+                           levels are work-bound and stay level-synchronous) */
 } mcm_options_t;
 
 typedef struct {
@@ -185,6 +193,7 @@ typedef struct {
   int64_t debug_violations;  /* consistency violations found by the debug checks (env MCM_DEBUG=1) */
   int64_t kernel_launches;   /* kernels launched by this handle's mcm_create plus by the last call (counted
                                 at the launch sites: the create's setup kernels + one persistent kernel) */
+  int64_t gr_window_levels;  /* BFS levels run inside windows (option gr_window; K per window) */
   double ms_init;            /* device time: initial matching + worklist build */
   double ms_gr;              /* device time in global relabels */
   double ms_loop;            /* device time in fix + push steps */

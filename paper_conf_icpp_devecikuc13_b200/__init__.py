@@ -65,6 +65,8 @@ class Options(ctypes.Structure):
         ("gr_target_min", ctypes.c_int32),
         ("gr_concurrent", ctypes.c_int32),
         ("perturb", ctypes.c_int32),
+        ("gr_window", ctypes.c_int32),
+        ("gr_window_max", ctypes.c_int32),
     ]
 
 
@@ -74,7 +76,7 @@ class Stats(ctypes.Structure):
     _fields_ = [(f, ctypes.c_int64) for f in (
         "loops", "gr_count", "gr_levels", "pushes", "blocked", "dead", "edges_scanned", "slots", "shrinks", "gaps",
         "guard_reactivated", "fixed_cols", "init_card", "card", "tail_loops", "grid_barriers", "gr_rows", "gr_edges",
-        "gr_cols", "greedy_edges", "rows_repaired", "tail_gr_levels", "debug_violations", "kernel_launches")] + [
+        "gr_cols", "greedy_edges", "rows_repaired", "tail_gr_levels", "debug_violations", "kernel_launches", "gr_window_levels")] + [
         (f, ctypes.c_double) for f in ("ms_init", "ms_gr", "ms_loop", "ms_total", "ms_setup")] + [
         ("grid_ctas", ctypes.c_int32), ("threads_per_cta", ctypes.c_int32)]
 

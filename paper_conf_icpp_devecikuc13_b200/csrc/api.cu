@@ -265,6 +265,8 @@ void mcm_default_options(mcm_options_t *o) {
   o->gr_target_min = 1024;
   o->tail_chain = 256;
   o->grid_chain = 128;
+  o->gr_window = 0;
+  o->gr_window_max = 16384;
 }
 
 static bool sizes_ok(int32_t m, int32_t n, int64_t nnz) {
@@ -301,6 +303,7 @@ static int check_opts(const mcm_options_t *o) {
   if (o->variant < 0 || o->variant > 1 || o->bu_div < 0 || o->tail_chain < 0 || o->grid_chain < 0) return MCM_EINVAL;
   if (o->gr_concurrent < 0 || o->gr_concurrent > MAX_CTAS) return MCM_EINVAL;
   if (o->perturb < 0 || o->perturb > 65536) return MCM_EINVAL;
+  if (o->gr_window < 0 || o->gr_window > 64 || o->gr_window_max < 0) return MCM_EINVAL;
   return MCM_OK;
 }
 
@@ -456,6 +459,8 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   p.variant = o.variant;
   p.tail_chain = o.tail_chain;
   p.perturb = o.perturb;
+  p.gr_window = o.gr_window;
+  p.gr_window_max = o.gr_window_max;
   // worklists of at most this many slots run as push chains (lanes per slot from the
   // count); MCM_CHAIN_SLOTS: analysis knob
   // (analysis knobs, clamped: 0..TW slots; a divisor of at least 1)
@@ -474,6 +479,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     p.gr_early = 0;
     p.compact_adapt = 0;
     p.compact_every = 0;
+    p.gr_window = 0;
   }
   p.tail_f = o.tail_f;
   p.max_loops = o.max_loops > 0 ? o.max_loops : 2LL * ((long long)h->m + h->n) + 100000;
@@ -491,7 +497,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   // the lean production instance unless a feature only the full one carries is on
   // (a cluster tail group spans several SMs' L1s: it needs gpu-scope vertex state)
   const bool conc = mode == MODE_SOLVE && o.gr_concurrent > 0 && !o.serial && !o.variant;
-  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1 || conc || o.perturb)
+  void (*kern)(const Params) = (mode != MODE_SOLVE || o.serial || o.variant || o.gap || p.debug || C > 1 || conc || o.perturb || o.gr_window > 1)
                                    ? gpr_kernel<F_ALL>
                                    : gpr_kernel<F_FAST>;
   if (o.grid_ctas > 0 && o.grid_ctas < C) C = 1;  // too few CTAs for a cluster: one-CTA tail group
@@ -582,6 +588,7 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
   s.gr_rows = x[ST_GR_ROWS]; s.gr_edges = x[ST_GR_EDGES]; s.gr_cols = x[ST_GR_COLS];
   s.greedy_edges = x[ST_GREEDY_EDGES]; s.rows_repaired = x[ST_REPAIRED]; s.tail_gr_levels = x[ST_TAIL_LEVELS];
   s.debug_violations = c.dbg[0];
+  s.gr_window_levels = x[ST_WINDOWS];
   s.kernel_launches = h->create_launches + 1;  // the create's kernels + this call's one persistent kernel
   s.ms_init = x[ST_NS_INIT] * 1e-6; s.ms_gr = x[ST_NS_GR] * 1e-6; s.ms_loop = x[ST_NS_LOOP] * 1e-6;
   s.ms_total = x[ST_NS_TOTAL] * 1e-6; s.ms_setup = h->ms_setup; s.grid_ctas = grid; s.threads_per_cta = NT;

@@ -66,7 +66,7 @@ enum {
   ST_LOOPS, ST_GRS, ST_LEVELS, ST_PUSHES, ST_BLOCKED, ST_DEAD, ST_SCANNED, ST_SLOTS, ST_SHRINKS, ST_GAPS,
   ST_GUARD, ST_FIXED, ST_INITCARD, ST_CARD, ST_TAILLOOPS, ST_BARRIERS, ST_NS_INIT, ST_NS_GR, ST_NS_LOOP,
   ST_NS_TOTAL, ST_MAXLEVEL, ST_REACHED_FREE, ST_GR_ROWS, ST_GR_EDGES, ST_GR_COLS, ST_GREEDY_EDGES, ST_TRACE_N, ST_REPAIRED,
-  ST_FLOOR_R, ST_FLOOR_C, ST_TAIL_LEVELS, ST_NSTAT = 32
+  ST_FLOOR_R, ST_FLOOR_C, ST_TAIL_LEVELS, ST_WINDOWS, ST_NSTAT = 32
 };
 
 struct Ctrl {
@@ -120,6 +120,7 @@ struct Params {
   int bu_div;              // bottom-up BFS level rule (see use_bottom_up; 0: top-down only)
   int scan_rot;            // push scans start at a (column, loop)-dependent rotation (tie-break)
   int perturb;             // fault injection: a push loses its row store with probability perturb/65536
+  int gr_window, gr_window_max;  // windowed GR levels (see gr_window_level): levels per window, frontier limit
   long long max_loops;
   // I/O
   const int *rmatch_in, *cmatch_in;
@@ -142,7 +143,8 @@ enum { SS_PUSH, SS_BLOCK, SS_DEAD, SS_SCAN, SS_SLOTS, SS_FREE, SS_GRROWS, SS_GRE
 // control-loop statistics and the phase-trace cursor: kept by the lead thread
 // (block 0, thread 0) only, in shared memory, so they hold no registers
 struct LeadStats {
-  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar, repaired, tail_levels;
+  long long grs, levels, shrinks, gaps, guard_re, loops, tail_loops, ns_gr, ns_loop, nbar, repaired, tail_levels,
+      wlevels;
   int tn, ttag, tsz, pad;
 };
 struct Smem;
@@ -163,6 +165,9 @@ struct Smem {
   u64 hugec[MAXHUGE];
   int huget[MAXHUGE];
   int nhuge;
+  int4 lq[2][512];         // windowed GR (option gr_window): the CTA's local BFS queues
+  int lqn[2];
+  int lwdirty, lwmax;
   u32 nd;                  // push: columns declared dead in this tile (-> Ctrl::ndead)
   int chmax;               // push_chain: longest chain of the phase
   int qcnt, qbase, tmp;
@@ -716,8 +721,8 @@ struct Solver {
         const int i0 = t + (int)threadIdx.x, i1 = i0 + NT;
         int4 q0 = i0 < curlen ? ld_q(cur4 + i0) : make_int4(-1, 0, 0, 0);
         int4 q1 = i1 < curlen ? ld_q(cur4 + i1) : make_int4(-1, 0, 0, 0);
-        if (q0.x >= 0) { S(SS_GRROWS) += !q0.w; S(SS_GREDGES) += q0.z - q0.y; }
-        if (q1.x >= 0) { S(SS_GRROWS) += !q1.w; S(SS_GREDGES) += q1.z - q1.y; }
+        if (q0.x >= 0) { S(SS_GRROWS) += !(q0.w & 1); S(SS_GREDGES) += q0.z - q0.y; }
+        if (q1.x >= 0) { S(SS_GRROWS) += !(q1.w & 1); S(SS_GREDGES) += q1.z - q1.y; }
         const bool big0 = q0.x >= 0 && q0.z - q0.y > BIG_DEG, big1 = q1.x >= 0 && q1.z - q1.y > BIG_DEG;
         expand_pair(big0 || q0.x < 0 ? 0 : q0.z - q0.y, q0.y, big1 || q1.x < 0 ? 0 : q1.z - q1.y, q1.y, lc, lr, next,
                     ncnt, guard, gcnt);
@@ -767,7 +772,7 @@ struct Solver {
         if (u >= 0) { s = ld_ro(p.rptr + u); e = ld_ro(p.rptr + u + 1); }
       } else if (i < curlen) {
         int4 q = ld_q(cur4 + i);
-        u = q.x; s = q.y; e = q.z; cont = q.w;
+        u = q.x; s = q.y; e = q.z; cont = q.w & 1;
       }
       if (GRID && lvl > 0 && MCM_FINE && t == cta<GRID>() * per_tile) tmark(102, 0);
       if (u >= 0 && gl == 0) { S(SS_GRROWS) += !cont; S(SS_GREDGES) += e - s; }
@@ -1012,7 +1017,9 @@ struct Solver {
   // The GR as a resumable state machine, so that a CTA-local GR (tail mode) can
   // hand a frontier that grew too wide over to the whole grid mid-BFS.
   struct GRState {
-    int lvl, deepest, nlen, cur_is_a, in_smem, reached, target, pad;  // reached/target: early stop (R22)
+    int lvl, deepest, nlen, cur_is_a, in_smem, reached, target, dirty;  // reached/target: early stop (R22)
+                                                                        // dirty: a window left labels below
+                                                                        // its end in the frontier
     long long fedges, visited;  // next frontier's adjacency entries; columns labelled in this GR
   };
   // level 0 (INITRELABEL + first expansion): U -> filtered U (in T, then swapped), frontier -> Qa
@@ -1056,6 +1063,199 @@ struct Solver {
       g.cur_is_a ^= 1;
     }
     return true;
+  }
+
+  // ---------------------------------------------------------------- windowed GR levels
+  // Option gr_window = K > 1 (a build addition; the paper's GR is level-synchronous,
+  // Alg. 5): K BFS levels per grid barrier.  Every CTA expands its share of the
+  // frontier (rows with label L0, entries carrying their label offset in .w, see
+  // below) and then, without leaving the CTA, the rows that share discovers, level
+  // after level (a shared-memory queue and CTA barriers), until every row it reached
+  // with a label below Lend = L0 + 2K is expanded; rows reached with label Lend form
+  // the next (global) frontier.  Because the CTAs run ahead of one another, a vertex
+  // can first be reached by a longer path: labels are lowered by CAS (a column's
+  // word, then its mate row's) and a row whose label was lowered is expanded again
+  // with the smaller label (label correcting).  When every CTA's queue is empty (the
+  // window's grid barrier) every vertex whose BFS distance is below Lend carries its
+  // exact distance (its shortest path's rows were each expanded with their exact
+  // label), and the frontier rows carry exactly Lend -- the state a level-synchronous
+  // BFS reaches after the level of L0 + 2K - 2, so the early stop (R22 / R28), the
+  // floors and maxLevel are as if the levels had run one by one.  A local queue that
+  // overflows sends its row to the global frontier with its own label (.w offset)
+  // and marks the window dirty: the next unit of GR work is then another window (its
+  // L0 = Lend decodes the offsets), and no stop test or hand-over happens before a
+  // clean window.  Frontier entry .w: bit 0 = continuation of a split row, the rest
+  // = L0 - label (0 for every entry of a level-synchronous frontier).
+  static constexpr int LQ = 512;
+  __device__ __forceinline__ bool lower_ok(u64 w, u32 l) const { return psi_of(w) < gr_base || psi_of(w) > l; }
+  // queue a row range for this CTA's next sub-level (label lab), or, when the queue
+  // is full, for the next window (dirty)
+  __device__ __forceinline__ void lpush(int4 x, int nb, int lab, int L0n, int4 *next, u32 *gcnt) {
+    cg::coalesced_group g = cg::coalesced_threads();
+    int b = 0;
+    if (g.thread_rank() == 0) b = atomicAdd(&sm.lqn[nb], (int)g.size());
+    b = g.shfl(b, 0) + (int)g.thread_rank();
+    if (b < LQ) {
+      x.w |= lab;
+      sm.lq[nb][b] = x;
+    } else {
+      x.w |= L0n - lab;
+      stage(x, next, gcnt);
+      sm.lwdirty = 1;
+    }
+  }
+  __device__ __forceinline__ void lpush_row(int w, int s, int e, int nb, int lab, int Lend, int4 *next, u32 *gcnt) {
+    for (int c = s; c < e || c == s; c += SPLIT) {
+      lpush(make_int4(w, c, min(e, c + SPLIT), c > s), nb, lab, Lend, next, gcnt);
+      if (e - s <= SPLIT) break;
+    }
+  }
+  // expand radj[j0, e) (stride `step`) of a row with label lab: columns get lab+1,
+  // their mates lab+2 (queued below Lend, staged at Lend)
+  __device__ __forceinline__ void expand_w(int j0, int e, int step, int lab, int Lend, int nb, int4 *next,
+                                           u32 *ncnt) {
+    const u32 lc = gr_base + (u32)lab + 1u, lr = lc + 1u;
+    for (int j = j0; j < e; j += step * KB) {
+      int v[KB], rs[KB], re[KB];
+      u64 cs[KB], old[KB], rw[KB];
+      bool won[KB];
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        int jj = j + k * step;
+        v[k] = jj < e ? ld_adj(p.radj + jj) : -1;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) cs[k] = v[k] >= 0 ? vld(p.colst + v[k]) : 0ull;
+#pragma unroll
+      for (int k = 0; k < KB; k++) {  // claim (lower) the column; the mate's word rides along
+        const bool try_ = v[k] >= 0 && lower_ok(cs[k], lc);
+        const int w = mu_of(cs[k]);
+        old[k] = try_ ? atomicCAS(p.colst + v[k], cs[k], pack(w, lc)) : ~cs[k];
+        const bool go = try_ && w >= 0;
+        rw[k] = go ? vld(p.rowst + w) : 0ull;
+        rs[k] = go ? ld_ro(p.rptr + w) : 0;
+        re[k] = go ? ld_ro(p.rptr + w + 1) : 0;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        won[k] = old[k] == cs[k];
+        if (!won[k] && v[k] >= 0 && old[k] != ~cs[k]) {  // lost a race: retry while still lower
+          u64 cur = old[k];
+          while (lower_ok(cur, lc)) {
+            const u64 o = atomicCAS(p.colst + v[k], cur, pack(mu_of(cur), lc));
+            if (o == cur) { won[k] = true; break; }
+            cur = o;
+          }
+          if (won[k]) {
+            cs[k] = cur;
+            const int w = mu_of(cur);
+            rw[k] = w >= 0 ? vld(p.rowst + w) : 0ull;
+            rs[k] = w >= 0 ? ld_ro(p.rptr + w) : 0;
+            re[k] = w >= 0 ? ld_ro(p.rptr + w + 1) : 0;
+          }
+        }
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) {  // lower the mate rows (all CASes in flight)
+        const int w = mu_of(cs[k]);
+        const bool mt = won[k] && w >= 0 && mu_of(rw[k]) == v[k];
+        old[k] = (mt && lower_ok(rw[k], lr)) ? atomicCAS(p.rowst + w, rw[k], pack(v[k], lr)) : ~rw[k];
+        if (won[k] && !mt) {  // an unmatched column (first label only: counted once)
+          if (psi_of(cs[k]) < gr_base) {
+            S(SS_FREE)++;
+            if (mu_of(cs[k]) != -2) count_free();
+          }
+        }
+        if (won[k] && psi_of(cs[k]) < gr_base) S(SS_GRCOLS)++;
+      }
+#pragma unroll
+      for (int k = 0; k < KB; k++) {
+        const int w = mu_of(cs[k]);
+        if (!(won[k] && w >= 0 && mu_of(rw[k]) == v[k])) continue;
+        bool low = old[k] == rw[k];
+        if (!low && old[k] != ~rw[k]) {
+          u64 cur = old[k];
+          while (lower_ok(cur, lr)) {
+            const u64 o = atomicCAS(p.rowst + w, cur, pack(v[k], lr));
+            if (o == cur) { low = true; break; }
+            cur = o;
+          }
+        }
+        if (!low) continue;
+        if (lab + 2 < Lend) {
+          lpush_row(w, rs[k], re[k], nb, lab + 2, Lend, next, ncnt);
+        } else {
+          stage_row(w, rs[k], re[k], next, ncnt);
+        }
+      }
+    }
+  }
+  // one entry (a row range with its label) by a lane group of G lanes; longer lists
+  // by the whole warp
+  __device__ __forceinline__ void win_entry(int4 q, bool ok, int lab, int G, int gl, int Lend, int nb, int4 *next,
+                                            u32 *ncnt, int &mx) {
+    const int lane = lane_id();
+    if (ok && gl == 0) { S(SS_GRROWS) += !(q.w & 1); S(SS_GREDGES) += q.z - q.y; }
+    if (ok) mx = max(mx, lab);
+    const bool big = ok && G < 32 && q.z - q.y > BIG_DEG;
+    if (ok && !big) expand_w(q.y + gl, q.z, G, lab, Lend, nb, next, ncnt);
+    unsigned bigm = __ballot_sync(0xffffffffu, big && gl == 0);
+    while (bigm) {
+      int bl = __ffs(bigm) - 1;
+      bigm &= bigm - 1;
+      int sb = __shfl_sync(0xffffffffu, q.y, bl), eb = __shfl_sync(0xffffffffu, q.z, bl);
+      int lb = __shfl_sync(0xffffffffu, lab, bl);
+      expand_w(sb + lane, eb, 32, lb, Lend, nb, next, ncnt);
+    }
+  }
+  // One window: the frontier cur4[0, curlen) (rows at L0, .w offsets) -> rows at
+  // Lend in `next`.  Ring counters: 0 next-frontier length (stage/flush), 2 alive
+  // unmatched columns labelled, 3 deepest expanded row label + 1, 4 next-frontier
+  // adjacency entries (fe_on), 5 rows expanded inside the window, 6 dirty.
+  __device__ void gr_window_level(const int4 *cur4, int curlen, int L0, int Lend, int4 *next, u32 *ncnt) {
+    if (threadIdx.x == 0) { sm.lqn[0] = 0; sm.lqn[1] = 0; sm.lwdirty = 0; sm.lwmax = 0; }
+    __syncthreads();
+    int mx = -1;
+    const int lane = lane_id();
+    {
+      const int G = pick_group(curlen, gridDim.x * NT);
+      const int gl = lane & (G - 1), per_tile = NT / G;
+      for (int t = blockIdx.x * per_tile; t < curlen; t += gridDim.x * per_tile) {
+        const int i = t + (int)threadIdx.x / G;
+        const bool ok = i < curlen;
+        int4 q = ok ? ld_q(cur4 + i) : make_int4(-1, 0, 0, 0);
+        win_entry(q, ok, L0 - (q.w & ~1), G, gl, Lend, 0, next, ncnt, mx);
+      }
+    }
+    int cb = 0, rows = 0, nr = 0;
+    for (;;) {
+      __syncthreads();
+      const int cnt = min(sm.lqn[cb], LQ);
+      if (cnt == 0) break;
+      rows += cnt;
+      __syncthreads();
+      if (threadIdx.x == 0) sm.lqn[cb ^ 1] = 0;
+      __syncthreads();
+      const int G = pick_group(cnt, NT);
+      const int gl = lane & (G - 1), per_tile = NT / G;
+      for (int t = 0; t < cnt; t += per_tile) {
+        const int i = t + (int)threadIdx.x / G;
+        const bool ok = i < cnt;
+        int4 q = ok ? sm.lq[cb][i] : make_int4(-1, 0, 0, 0);
+        win_entry(q, ok, q.w & ~1, G, gl, Lend, cb ^ 1, next, ncnt, mx);
+      }
+      cb ^= 1;
+      nr++;
+    }
+    mx = __reduce_max_sync(0xffffffffu, mx);
+    if (lane == 0 && mx >= 0) atomicMax(&sm.lwmax, mx + 1);
+    flush(next, ncnt);  // (its barriers order the lwmax updates before thread 0 reads it)
+    if (threadIdx.x == 0) {
+      if (sm.lwmax) atomicMax(ring_now(3), (u32)sm.lwmax);
+      if (rows) atomicAdd(ring_now(5), (u32)rows);
+      if (sm.lwdirty) atomicAdd(ring_now(6), 1u);
+      if (p.trace && nr) atomicMax(ring_now(7), (u32)nr);
+    }
   }
 
   // ---------------------------------------------------------------- fix step
@@ -1392,17 +1592,24 @@ struct Solver {
       // behind the next column's loads): {column, row, expected, written, returned}
       int pc = -1, pr = -1;
       u64 pexp = 0, pnew = 0, pret = 0;
+      // the next column's word and adjacency bounds, loaded by the group's lead lane
+      // in the same round trip as the row claim (the displaced column is known from
+      // the scan): one dependent round trip less per push
+      bool have = false;
+      u64 ncs = 0;
+      int ns = 0, ne = 0;
       while (cur >= 0) {
         if (step >= cap || retry > 8) { left = cur; break; }
-        const u64 cs = vld(p.colst + cur);
+        const u64 cs = have ? ncs : vld(p.colst + cur);
         const int psiv = labf(psi_of(cs), base, fl_c);
-        const int s = ld_ro(p.cptr + cur);
-        int e = ld_ro(p.cptr + cur + 1);
+        const int s = have ? ns : ld_ro(p.cptr + cur);
+        int e = have ? ne : ld_ro(p.cptr + cur + 1);
+        have = false;
         if (p.dead_skip && psiv >= INF) e = s;  // R19
         if (step > 0 && e - s > HUGE_DEG * G / 32) { left = cur; break; }  // a long list ends the chain
-        u64 best;
+        u64 best, braw = 0;
         int ub, wb;
-        scan(s, e, gl, G, gmask, psiv - 1, base, best, ub, wb, 0, retry > 0);  // l.4-11
+        scan(s, e, gl, G, gmask, psiv - 1, base, best, ub, wb, 0, retry > 0, &braw);  // l.4-11
         if (gl == 0 && pc >= 0) { chain_settle(pc, pr, pexp, pnew, pret); pc = -1; }
         const int psimin = best == ~0ull ? INF : (int)(best >> 32);
         if (psimin >= INF) {  // l.19-22: dead
@@ -1415,9 +1622,10 @@ struct Solver {
         }
         int ok = 0;
         if (gl == 0) {
-          const u64 now = ld_rlx(p.rowst + ub);  // gpu scope: L2's current word
-          if (mu_of(now) == wb && labf(psi_of(now), base, fl_r) == psimin)
-            ok = atomicCAS(p.rowst + ub, now, pack(cur, base + (u32)psimin + 2u)) == now;  // l.14, l.17
+          if (wb >= 0) { ncs = vld(p.colst + wb); ns = ld_ro(p.cptr + wb); ne = ld_ro(p.cptr + wb + 1); }
+          // claim the row against the word the scan read (gpu scope): it fails when
+          // any push changed the row since
+          ok = atomicCAS(p.rowst + ub, braw, pack(cur, base + (u32)psimin + 2u)) == braw;  // l.14, l.17
           if (ok) {  // l.15, l.16
             pc = cur; pr = ub; pexp = cs; pnew = pack(ub, base + (u32)psimin + 1u);
 #if MCM_CHAIN_PLAIN  // A/B only: the plain store of the first round-1 build
@@ -1433,6 +1641,10 @@ struct Solver {
         retry = 0;
         step++;
         cur = wb;  // -1: single push, the path is complete
+        ncs = __shfl_sync(gmask, ncs, lead_lane);
+        ns = __shfl_sync(gmask, ns, lead_lane);
+        ne = __shfl_sync(gmask, ne, lead_lane);
+        have = true;
       }
       __syncwarp(gmask);  // every lane of the group has read Ac(i) before it is cleared
       if (gl == 0) {
@@ -1515,8 +1727,9 @@ struct Solver {
   // free tie-break in parallel mode, R11: contenders for one low-label row spread
   // over the equally low rows instead of blocking each other)
   // fresh: row words at gpu scope (L2), for a push chain re-scanning after a lost CAS
+  // raw (optional): the winner's row word as the scan read it (push chains CAS against it)
   __device__ __forceinline__ void scan(int s, int e, int gl, int G, unsigned gmask, int target, u32 base, u64 &best,
-                                       int &bu, int &bw, int rot = 0, bool fresh = false) {
+                                       int &bu, int &bw, int rot = 0, bool fresh = false, u64 *raw = nullptr) {
     best = ~0ull;
     bu = -1;
     bw = -1;
@@ -1533,7 +1746,7 @@ struct Solver {
       }
 #pragma unroll
       for (int k = 0; k < KB; k++) rs[k] = x[k] >= 0 ? (fresh ? ld_rlx(p.rowst + x[k]) : vld(p.rowst + x[k])) : 0ull;
-      u64 key = ~0ull;
+      u64 key = ~0ull, kr = 0;
       int kx = -1, kw = -1;
 #pragma unroll
       for (int k = 0; k < KB; k++) {
@@ -1541,7 +1754,7 @@ struct Solver {
         S(SS_SCAN)++;
         int l = labf(psi_of(rs[k]), base, fl_r);
         u64 kk = l < INF ? (((u64)(u32)l << 32) | (u32)(c0 + gl + k * G - s)) : ~0ull;
-        if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); }
+        if (kk < key) { key = kk; kx = x[k]; kw = mu_of(rs[k]); kr = rs[k]; }
       }
       u64 km = key;
       for (int o = G >> 1; o > 0; o >>= 1) {
@@ -1553,6 +1766,7 @@ struct Solver {
         best = km;
         bu = __shfl_sync(gmask, kx, src);
         bw = __shfl_sync(gmask, kw, src);
+        if (raw) *raw = __shfl_sync(gmask, kr, src);
       }
       if (best != ~0ull && (int)(best >> 32) == target) break;
     }
@@ -1712,6 +1926,11 @@ struct Solver {
   // the grid when a frontier outgrows it, back to the tail below tail_f()/2)
   __device__ __forceinline__ bool early_gr() const { return p.gr_early && !p.gap; }
   __device__ __forceinline__ int tail_f() const { return p.tail_f > 0 ? p.tail_f : 2 * p.tail_max; }
+  // the next GR unit is a window (gr_window_step) rather than one level
+  __device__ __forceinline__ bool win_ok(const Ctl &c) const {
+    return (F & F_AUX) && p.gr_window > 1 && (c.gst.dirty || (c.gst.nlen <= p.gr_window_max && !c.gst.in_smem &&
+                                               !use_bottom_up(c.gst.fedges, (long long)n - c.gst.visited, c.gst.nlen)));
+  }
 
   // ---------------------------------------------------------------- units of work
   // Single-CTA tail GR levels keep the frontier in shared memory: stage() writes
@@ -1836,6 +2055,35 @@ struct Solver {
     if (g.nlen == 0) gr_finish(c);
     else if (g.reached >= g.target) gr_finish(c, true);
     if (GRID && MCM_FINE) tmark(106, 0);
+    if (lead()) L().ns_gr += (long long)(tnow() - g0);
+  }
+  // K BFS levels in one grid phase (option gr_window; see gr_window_level)
+  __device__ void gr_window_step(Ctl &c) {
+    u64 g0 = tnow();
+    GRState &g = c.gst;
+    g.lvl += 2;  // the frontier's label L0
+    const int L0 = g.lvl, Lend = L0 + 2 * p.gr_window;
+    const int4 *cur = Q4(g.cur_is_a ? 0 : 1);
+    int4 *nxt = Q4(g.cur_is_a ? 1 : 0);
+    gr_base = c.base;
+    trace(5, g.nlen);
+    set_fe(g.nlen);
+    gr_window_level(cur, g.nlen, L0, Lend, nxt, ring_now(0));
+    barrier<true>();
+    g.fedges = ring_prev(4);
+    g.nlen = (int)ring_prev(0);
+    g.in_smem = 0;
+    g.reached += (int)ring_prev(2);
+    g.visited += (long long)g.nlen + ring_prev(2) + ring_prev(5);
+    const int mx = (int)ring_prev(3) - 1;  // deepest row label expanded
+    if (mx > g.deepest) g.deepest = mx;
+    g.dirty = ring_prev(6) != 0;
+    g.lvl = Lend - 2;  // (clean) every row below Lend expanded, the frontier holds Lend
+    g.cur_is_a ^= 1;
+    if (lead()) L().wlevels += p.gr_window;
+    if (p.trace) { tmark(150, (int)ring_prev(7)); tmark(151, (int)ring_prev(5)); tmark(152, g.dirty); }
+    if (g.nlen == 0) gr_finish(c);
+    else if (!g.dirty && g.reached >= g.target) gr_finish(c, true);
     if (lead()) L().ns_gr += (long long)(tnow() - g0);
   }
   // SHRKRNL: the fix step of every slot (fix_slots, Alg. 8) with the
@@ -2308,7 +2556,7 @@ struct Solver {
       }
       const int up = tail_f();
       bool tail_ok = p.tail_max > 0 &&
-                     (c.gr_active ? c.gst.nlen <= up / 2
+                     (c.gr_active ? (c.gst.nlen <= up / 2 && !c.gst.dirty)
                                   : (c.loop == c.gapAt ? false
                                                        : (c.loop == c.iterGR ? (c.ulen <= up && !base_overflow(c))
                                                                              : c.len <= p.tail_max)));
@@ -2325,7 +2573,11 @@ struct Solver {
         continue;
       }
       // one unit of grid work
-      if (c.gr_active) { gr_step<true>(c); continue; }                // Alg. 5 level
+      if (c.gr_active) {                                               // Alg. 5 level(s)
+        if (win_ok(c)) gr_window_step(c);
+        else gr_step<true>(c);
+        continue;
+      }
       if ((F & F_GAP) && c.loop == c.gapAt) {                          // gap relabel (R14)
         u64 g0 = tnow();
         if (gap_relabel(c.base - stride()) >= 0 && lead()) L().gaps++;
@@ -2368,8 +2620,9 @@ struct Solver {
     const int up = tail_f();
     for (;;) {
       if (!c.gr_active && c.loop != c.iterGR) break;  // gr_finish moved iterGR past loop: done
-      const bool tail_ok = p.tail_max > 0 && (c.gr_active ? c.gst.nlen <= up / 2 : c.ulen <= up);
+      const bool tail_ok = p.tail_max > 0 && (c.gr_active ? (c.gst.nlen <= up / 2 && !c.gst.dirty) : c.ulen <= up);
       if (tail_ok) tail_episode(c);
+      else if (c.gr_active && win_ok(c)) gr_window_step(c);
       else if (c.gr_active) gr_step<true>(c);
       else gr_begin<true>(c);
     }
@@ -2630,6 +2883,7 @@ struct Solver {
       st[ST_BARRIERS] = l.nbar;
       st[ST_REPAIRED] = l.repaired;
       st[ST_TAIL_LEVELS] = l.tail_levels;
+      st[ST_WINDOWS] = l.wlevels;
       st[ST_TRACE_N] = l.tn;
       if (p.mode == MODE_SOLVE || p.mode == MODE_INIT) {
         st[ST_CARD] = (long long)ring_prev(0);

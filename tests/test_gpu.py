@@ -119,6 +119,7 @@ OPTION_SETS = [
     dict(gr_target=0.3, k=0.3, gr_target_min=0), dict(gr_target=0.01, tail_max=0, gr_target_min=16),
     dict(gr_concurrent=48), dict(gr_concurrent=16, k=3.0), dict(gr_concurrent=100, tail_max=0),
     dict(gr_concurrent=1, grid_chain=0, tail_chain=0),
+    dict(gr_window=4), dict(gr_window=8, gr_window_max=1 << 30, tail_max=0), dict(gr_window=16, k=0.1),
 ]
 
 

@@ -189,7 +189,13 @@ def _matchings(g, rng):
 
 
 TAIL_OPTS = [dict(tail_max=32, tail_f=128), dict(tail_max=32, tail_f=8), dict(tail_max=32, tail_f=100000),
-             dict(tail_max=32, tail_f=4, bu_div=0), dict(tail_max=0)]
+             dict(tail_max=32, tail_f=4, bu_div=0), dict(tail_max=0),
+             # windowed levels (R29): K levels per grid barrier, label-correcting inside a CTA;
+             # gr_window_max 2^30 also sends wide levels through windows (local-queue overflow ->
+             # dirty windows)
+             dict(tail_max=32, tail_f=128, gr_window=4), dict(tail_max=0, gr_window=8, gr_window_max=1 << 30),
+             dict(tail_max=32, tail_f=8, gr_window=2, gr_window_max=64, bu_div=0),
+             dict(tail_max=0, gr_window=64, gr_window_max=1 << 30, bu_div=0)]
 
 
 @pytest.mark.parametrize("oi", range(len(TAIL_OPTS)))
@@ -218,7 +224,9 @@ def test_relabel_tail_paths_bit_exact(gi, oi):
 
 
 EARLY_OPTS = [dict(gr_target=1.0), dict(gr_target=0.6, gr_target_min=0), dict(gr_target=0.3, gr_target_min=0, tail_max=0),
-              dict(gr_target=0.05, gr_target_min=16, tail_f=16)]
+              dict(gr_target=0.05, gr_target_min=16, tail_f=16),
+              dict(gr_target=1.0, gr_window=4), dict(gr_target=0.3, gr_target_min=0, tail_max=0, gr_window=8,
+                                                     gr_window_max=1 << 30)]
 
 
 @pytest.mark.parametrize("oi", range(len(EARLY_OPTS)))

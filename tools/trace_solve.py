@@ -11,11 +11,16 @@ import torch  # noqa: E402
 import synth  # noqa: E402
 import paper_conf_icpp_devecikuc13_b200 as pkg  # noqa: E402
 
-TAGS = {1: "gr_level0", 2: "gr_level", 3: "fix", 4: "push", 0: "other"}
+TAGS = {1: "gr_level0", 2: "gr_level", 3: "fix", 4: "push", 5: "gr_window", 0: "other"}
 
 
 def summarize(path):
     t = np.fromfile(path, dtype=np.int64).reshape(-1, 3)
+    for tag, what in ((150, "window: most local rounds of a CTA"), (151, "window: rows expanded inside"),
+                      (152, "window: dirty")):
+        x = t[t[:, 0] == tag, 1]
+        if x.size:
+            print(f"{what}: n={x.size} mean={x.mean():.2f} p50={np.median(x):.0f} max={x.max()}")
     d = np.diff(t[:, 2]) / 1e3  # us; phase i ends at record i+1? record i = end of phase with tag t[i]
     keep = t[:, 0] < 100  # drop intra-phase marks from the per-phase summary
     t = t[keep]
