@@ -2081,6 +2081,21 @@ struct Solver {
     g.lvl = Lend - 2;  // (clean) every row below Lend expanded, the frontier holds Lend
     g.cur_is_a ^= 1;
     if (lead()) L().wlevels += p.gr_window;
+    if (g.nlen == 0) {
+      // the BFS ended inside this window: a row expanded with a label that was
+      // lowered later makes mx too large, so maxLevel comes from the final labels
+      // (one pass over the rows; at most once per GR)
+      const u32 b = c.base;
+      u32 best = 0;
+      for (long long u = (long long)blockIdx.x * NT + threadIdx.x; u < m; u += (long long)gridDim.x * NT) {
+        const u32 ps = psi_of(vld(p.rowst + u));
+        if (ps >= b && ps - b + 1u > best) best = ps - b + 1u;
+      }
+      best = __reduce_max_sync(0xffffffffu, best);
+      if (lane_id() == 0 && best) atomicMax(ring_now(3), best);
+      barrier<true>();
+      g.deepest = (int)ring_prev(3) - 1;
+    }
     if (p.trace) { tmark(150, (int)ring_prev(7)); tmark(151, (int)ring_prev(5)); tmark(152, g.dirty); }
     if (g.nlen == 0) gr_finish(c);
     else if (!g.dirty && g.reached >= g.target) gr_finish(c, true);
