@@ -52,6 +52,10 @@ def test_host_only_calls():
     assert L.mcm_match_host(None, None, 4, 4, 0, None, 0, None, None, None, None, None) == -1
     assert L.mcm_destroy(None) == -1
     assert L.mcm_set_k(None, 0.5) == -1
+    L.mcm_pgr_init.restype = ctypes.c_int
+    L.mcm_pgr_level.restype = ctypes.c_int
+    assert L.mcm_pgr_init(None, None, 1, 0, 1, None, None, None, None) == -1
+    assert L.mcm_pgr_level(None, None, 1, 0, 1, 0, None, None, None, None, None, None, None) == -1
     h = ctypes.c_void_p()
     assert L.mcm_create(None, None, 4, 4, 0, None, 0, None, None, ctypes.byref(h)) == -1
     assert pkg.mcm_default_options().gr_target == 0.6 and pkg.mcm_default_options().gr_target_min == 1024

@@ -19,15 +19,15 @@ if len(sys.argv) > 4:
         opts[k] = float(v) if "." in v else int(v)
 g = synth.config(name)
 mt = pkg.Matcher(torch.from_numpy(g.indptr).cuda(), torch.from_numpy(g.indices).cuda(), g.m, g.n, **opts)
-ts, lv, lp, gr, lm, pu = [], [], [], [], [], []
+ts, lv, lp, gr, lm, pu, im = [], [], [], [], [], [], []
 for r in range(reps + 1):
     card, _, _ = mt.solve()
     st = mt.stats()
     assert card == st["card"]
     if r:
         ts.append(st["ms_total"]); lv.append(st["gr_levels"]); lp.append(st["loops"]); gr.append(st["ms_gr"])
-        lm.append(st["ms_loop"]); pu.append(st["pushes"])
+        lm.append(st["ms_loop"]); pu.append(st["pushes"]); im.append(st["ms_init"])
 print(f"{label:10s} {name} card={card} ms med={statistics.median(ts):.2f} mean={statistics.mean(ts):.2f} "
       f"min={min(ts):.2f} max={max(ts):.2f} gr_ms med={statistics.median(gr):.2f} levels med={statistics.median(lv)} "
-      f"loops med={statistics.median(lp)} loop_ms med={statistics.median(lm):.2f} us/push(loop) "
+      f"loops med={statistics.median(lp)} init_ms med={statistics.median(im):.3f} loop_ms med={statistics.median(lm):.2f} us/push(loop) "
       f"{1e3 * sum(lm) / max(1, sum(pu)):.3f}", flush=True)
