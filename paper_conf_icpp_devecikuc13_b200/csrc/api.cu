@@ -446,6 +446,15 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     if ((size_t)tcap > room) tcap = (int)room;
     p.trace = (long long *)(ws + L.dbg);
     p.trace_cap = tcap;
+    // MCM_CTATIME=<phases> (with MCM_TRACE): every CTA's arrival time at the grid
+    // barriers of the first <phases> phases, after the trace records; dumped to
+    // MCM_CTATIME_FILE (analysis of load imbalance only, tools/cta_imbalance.py)
+    const int cn = getenv("MCM_CTATIME") ? atoi(getenv("MCM_CTATIME")) : 0;
+    const size_t left = (h->L.total - h->L.dbg) / sizeof(long long) - 3 * (size_t)tcap;
+    if (cn > 0 && h->max_grid > 0) {
+      p.ctat = p.trace + 3 * (size_t)tcap;
+      p.ctat_n = (int)std::min<size_t>((size_t)cn, left / (size_t)h->max_grid);
+    }
   }
   const mcm_options_t &o = h->opt;
   p.k = o.k; p.gr_fixed = o.gr_strategy == MCM_GR_FIXED; p.shrink_min = o.shrink_min; p.init = o.init;
@@ -601,6 +610,17 @@ static int64_t launch(mcm_ctx *h, cudaStream_t st, int mode, const int32_t *rin,
     cudaMemcpy(buf.data(), p.trace, buf.size() * sizeof(long long), cudaMemcpyDeviceToHost);
     FILE *f = fopen(getenv("MCM_TRACE_FILE"), "wb");
     if (f) { fwrite(buf.data(), sizeof(long long), buf.size(), f); fclose(f); }
+  }
+  if (p.ctat && getenv("MCM_CTATIME_FILE")) {
+    std::vector<long long> buf((size_t)p.ctat_n * h->grid);
+    cudaMemcpy(buf.data(), p.ctat, buf.size() * sizeof(long long), cudaMemcpyDeviceToHost);
+    FILE *f = fopen(getenv("MCM_CTATIME_FILE"), "wb");
+    if (f) {
+      const long long hdr[2] = {p.ctat_n, h->grid};
+      fwrite(hdr, sizeof(long long), 2, f);
+      fwrite(buf.data(), sizeof(long long), buf.size(), f);
+      fclose(f);
+    }
   }
   if (c.err) return c.err;
   if (mode == MODE_RELABEL || mode == MODE_GAP || mode == MODE_UNIT) return x[ST_MAXLEVEL];

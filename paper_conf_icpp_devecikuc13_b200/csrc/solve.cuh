@@ -105,6 +105,8 @@ struct Params {
   int hist_len;
   int debug;
   long long *trace;        // optional phase trace: {tag, size, t_end_ns} triples (MCM_TRACE)
+  long long *ctat;         // optional: per-CTA grid-barrier arrival times [phase][cta] (MCM_CTATIME)
+  int ctat_n;
   int trace_cap;
   Ctrl *ctrl;
   // options
@@ -249,6 +251,10 @@ struct Solver {
     };
     if (GRID) {
       if (MCM_FINE) tmark(105, 0);
+      if (p.ctat) {  // analysis only: when the CTA's last warp reached this barrier
+        __syncthreads();
+        if (threadIdx.x == 0 && ph < p.ctat_n) p.ctat[(long long)ph * gridDim.x + blockIdx.x] = (long long)gtime();
+      }
       if (RP) grid_sync(&p.ctrl->bar, false, load_rp);
       else grid_sync(&p.ctrl->bar, false);
       if (lead()) L().nbar++;
