@@ -555,11 +555,25 @@ struct Solver {
       }
       int u[RG][KB];
       u64 rs[RG][KB];
+      // lists longer than KB: the first KB candidates start at a column-dependent
+      // rotation of Gamma(v) (reading R13), so the first claims of R-MAT columns,
+      // whose lists all begin with the same few hub rows, spread over their rows; a
+      // column whose candidates were all taken then walks its whole list from s
+      int rot[RG];
+#pragma unroll
+      for (int k = 0; k < RG; k++) {
+        const int d = e[k] - s[k];
+        rot[k] = d > KB ? (int)(((u32)v[k] * 2654435761u) % (u32)d) : 0;
+      }
 #pragma unroll
       for (int k = 0; k < RG; k++)
 #pragma unroll
-        for (int q = 0; q < KB; q++)
-          u[k][q] = s[k] + q < e[k] ? ld_adj(p.cadj + s[k] + q) : -1;
+        for (int q = 0; q < KB; q++) {
+          const int d = e[k] - s[k];
+          int x = rot[k] + q;
+          if (x >= d) x -= d;
+          u[k][q] = q < d ? ld_adj(p.cadj + s[k] + x) : -1;
+        }
 #pragma unroll
       for (int k = 0; k < RG; k++)
 #pragma unroll
@@ -581,7 +595,7 @@ struct Solver {
 #pragma unroll
         for (int q = 0; q < KB; q++)
           if (q == pick) { cu[k] = u[k][q]; exp_[k] = rs[k][q]; }
-        pos[k] = pick >= 0 ? s[k] + pick + 1 : s[k] + KB;
+        pos[k] = rot[k] ? s[k] : (pick >= 0 ? s[k] + pick + 1 : s[k] + KB);
       }
 #pragma unroll
       for (int k = 0; k < RG; k++)
