@@ -315,13 +315,16 @@ struct Solver {
   // skip_iso: columns without any edge are left out as well (returns their count):
   // they can never be matched, and a first push would only declare them dead
   template <int RB>
-  __device__ __forceinline__ int cols_unmatched(int i0, int hi, int *val, bool skip_iso) const {
+  // consistent: every matched column's row points back (the device greedy's M0:
+  // its row CAS precedes the column store), so R1 needs no row-word load
+  __device__ __forceinline__ int cols_unmatched(int i0, int hi, int *val, bool skip_iso, bool consistent) const {
     u64 cw[RB], rw[RB];
     int cs[RB], ce[RB];
 #pragma unroll
     for (int k = 0; k < RB; k++) cw[k] = i0 + k < hi ? vld(p.colst + i0 + k) : pack(-2, 0);
 #pragma unroll
-    for (int k = 0; k < RB; k++) rw[k] = mu_of(cw[k]) >= 0 ? vld(p.rowst + mu_of(cw[k])) : 0ull;
+    for (int k = 0; k < RB; k++)
+      rw[k] = (!consistent && mu_of(cw[k]) >= 0) ? vld(p.rowst + mu_of(cw[k])) : pack(i0 + k, 0);
 #pragma unroll
     for (int k = 0; k < RB; k++) {
       const bool f = skip_iso && mu_of(cw[k]) == -1;
@@ -2542,8 +2545,9 @@ struct Solver {
     const bool skip_iso = (p.mode == MODE_SOLVE || p.mode == MODE_RELABEL) && !((F & F_SERIAL) && p.serial) &&
                           !((F & F_FIRST) && p.variant == 1);
     long long iso_c = 0;
+    const bool consistent = p.mode == MODE_SOLVE && p.init == 0;  // M0 from the device greedy
     int run1 = compact_pass1<true, 8>(
-        n, [&](int i0, int hi, int *val) { iso_c += cols_unmatched<8>(i0, hi, val, skip_iso); }, T, Ac);
+        n, [&](int i0, int hi, int *val) { iso_c += cols_unmatched<8>(i0, hi, val, skip_iso, consistent); }, T, Ac);
     iso_c = cta_sum<NT>(iso_c, sm.red);
     if (threadIdx.x == 0 && iso_c) atomicAdd(&p.ctrl->ndead, (u32)iso_c);
     barrier<true>();
