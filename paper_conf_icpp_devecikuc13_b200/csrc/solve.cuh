@@ -1660,11 +1660,7 @@ struct Solver {
             S(SS_PUSH)++;
           }
         }
-        if (!__shfl_sync(gmask, ok, lead_lane)) {  // the row changed: scan again
-          retry++;
-          if (GRID && p.trace && gl == 0) atomicAdd(ring_now(3), 1u);  // (trace only: lost claims)
-          continue;
-        }
+        if (!__shfl_sync(gmask, ok, lead_lane)) { retry++; continue; }  // the row changed: scan again
         retry = 0;
         step++;
         cur = wb;  // -1: single push, the path is complete
@@ -2193,7 +2189,7 @@ struct Solver {
     if (chain_grid || poll) {
       barrier<GRID, true>();
       if (chain_grid) adv = max(1, (int)ring_prev(5));
-      if (chain_grid && p.trace) { tmark(160, (int)ring_prev(5)); tmark(161, (int)ring_prev(3)); }
+      if (chain_grid && p.trace) tmark(160, (int)ring_prev(5));
       if (poll && ring_prev(6)) c.cflags |= 2;
     } else {
       barrier<GRID, false>();

@@ -17,8 +17,7 @@ TAGS = {1: "gr_level0", 2: "gr_level", 3: "fix", 4: "push", 5: "gr_window", 0: "
 def summarize(path):
     t = np.fromfile(path, dtype=np.int64).reshape(-1, 3)
     for tag, what in ((150, "window: most local rounds of a CTA"), (151, "window: rows expanded inside"),
-                      (152, "window: dirty"), (160, "grid chain phase: longest chain (pushes)"),
-                      (161, "grid chain phase: lost claims")):
+                      (152, "window: dirty"), (160, "grid chain phase: longest chain (pushes)")):
         x = t[t[:, 0] == tag, 1]
         if x.size:
             print(f"{what}: n={x.size} mean={x.mean():.2f} p50={np.median(x):.0f} max={x.max()}")
