@@ -75,18 +75,19 @@ def _graph(name, rank):
 
     if name == "C5":
         return synth.config("C5", 1.0, index=rank)
-    g = synth.config(name)
     if rank == 0:
-        return g
-    # an independent instance of the same recipe for rank > 0 (same distribution)
-    if name == "C1":
-        return synth.uniform(g.m, g.n, 8 * g.m, 1 + 7919 * rank, name="C1")
-    if name == "C2":
-        return synth.banded(g.n, 2.47, 64, 150, 2000, 2 + 7919 * rank, True, name="C2")
+        return synth.config(name)
+    # an independent instance of the same recipe for rank > 0 (same distribution);
+    # the large recipes are generated once, not after rank 0's graph as well
     if name == "C3":
         return synth.road(4900, 0.5, 0.4, 0.1, 3 + 7919 * rank, True, False, 256, name="C3")
     if name == "C4":
         return synth.rmat(23, 16 << 23, seed=4 + 7919 * rank, name="C4")
+    g = synth.config(name)
+    if name == "C1":
+        return synth.uniform(g.m, g.n, 8 * g.m, 1 + 7919 * rank, name="C1")
+    if name == "C2":
+        return synth.banded(g.n, 2.47, 64, 150, 2000, 2 + 7919 * rank, True, name="C2")
     raise KeyError(name)
 
 
